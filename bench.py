@@ -1,0 +1,397 @@
+#!/usr/bin/env python
+"""bench.py -- GCUPS of the B200 wavefront sweep (BASELINE.json metric) on BASELINE configs.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference] [--config C4]
+
+One "step" = one pass of the whole hot path (one wf_run over the full grid; every §8(a)
+row) with inputs already resident in HBM.  N>1 is launched by torchrun (one rank per GPU,
+column slabs, NVLink P2P edge exchange); timing is CUDA events on the launching stream,
+max over ranks.  Rank 0 prints ONE JSON line.
+
+--impl reference times the CPU oracle (the repo's stated reference arm for this tier) on a
+bounded row-prefix sample of the same workload, on this host's cores.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import workloads  # noqa: E402
+
+METRIC = "GCUPS (cell updates/sec) at 1/2/4/8 B200 and % of HBM roofline"
+UNIT = "GCUPS"
+L2_BYTES = 126 * 2 ** 20
+
+
+def _env_int(name, default):
+    v = os.environ.get(name)
+    return int(v) if v not in (None, "") else default
+
+
+def load_peaks():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            pk = json.load(f)
+        return float(pk["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs, copy read+write)"
+    except Exception:
+        return 6650.0, "fallback (B200_PROFILING.md 6.65 TB/s)"
+
+
+def load_traffic(workload_key):
+    try:
+        with open(os.path.join(ROOT, "profiles", "ncu_traffic.json")) as f:
+            return json.load(f).get(workload_key)
+    except Exception:
+        return None
+
+
+class ClockSampler:
+    """SM clocks and throttle reasons DURING the timed region (NVML, 10 ms period)."""
+
+    REASONS = {0x1: "gpu_idle", 0x2: "applications_clocks_setting", 0x4: "sw_power_cap", 0x8: "hw_slowdown",
+               0x10: "sync_boost", 0x20: "sw_thermal_slowdown", 0x40: "hw_thermal_slowdown",
+               0x80: "hw_power_brake_slowdown", 0x100: "display_clock_setting"}
+
+    def __init__(self, device_index):
+        self.samples, self.reasons, self.max_mhz = [], set(), None
+        self._stop = threading.Event()
+        self._thr = None
+        try:
+            import pynvml
+            pynvml.nvmlInit()
+            self._nv = pynvml
+            self._h = pynvml.nvmlDeviceGetHandleByIndex(device_index)
+            self.max_mhz = pynvml.nvmlDeviceGetMaxClockInfo(self._h, pynvml.NVML_CLOCK_SM)
+        except Exception:
+            self._nv = None
+
+    def _run(self):
+        nv = self._nv
+        while not self._stop.is_set():
+            try:
+                self.samples.append(nv.nvmlDeviceGetClockInfo(self._h, nv.NVML_CLOCK_SM))
+                r = nv.nvmlDeviceGetCurrentClocksEventReasons(self._h)
+                for bit, name in self.REASONS.items():
+                    if r & bit and name != "gpu_idle":
+                        self.reasons.add(name)
+            except Exception:
+                pass
+            time.sleep(0.01)
+
+    def __enter__(self):
+        if self._nv:
+            self._thr = threading.Thread(target=self._run, daemon=True)
+            self._thr.start()
+        return self
+
+    def __exit__(self, *a):
+        self._stop.set()
+        if self._thr:
+            self._thr.join()
+
+    def summary(self):
+        if not self.samples:
+            return {"sm_mhz": None, "sm_max_mhz": self.max_mhz, "reasons": ["unavailable"]}
+        return {"sm_mhz": statistics.median(self.samples), "sm_max_mhz": self.max_mhz,
+                "reasons": sorted(self.reasons), "samples": len(self.samples)}
+
+
+def host_inputs(cfg):
+    if cfg.fn == "seqcmp":
+        return workloads.seqcmp_inputs(cfg.dim)
+    if cfg.fn == "synthetic":
+        return workloads.synthetic_inputs(cfg.dim, cfg.dim, cfg.dsize)
+    return workloads.nash_inputs(cfg.dim, cfg.dim)
+
+
+def fn_kwargs(cfg):
+    kw = {}
+    if cfg.fn == "synthetic":
+        kw = dict(tsize=cfg.tsize, dsize=cfg.dsize)
+    elif cfg.fn == "nash":
+        kw = dict(tsize=cfg.tsize, dsize=4)
+    return kw
+
+
+# ------------------------------------------------------------------------------------ oracle arm
+def oracle_sample(cfg, inputs, rows):
+    """Run the oracle on the exact row prefix 1..rows (full width); returns seconds."""
+    import oracle
+    t0 = time.perf_counter()
+    if cfg.fn == "seqcmp":
+        x, y = inputs
+        oracle.seqcmp(x, y, m_compute=rows, out=_scratch_grid(cfg))
+    elif cfg.fn == "synthetic":
+        u, v, top, left = inputs
+        oracle.synthetic(u, v, top, left, cfg.tsize, m_compute=rows)
+    else:
+        r, c, top, left = inputs
+        oracle.nash(r, c, top, left, nstrat=cfg.tsize, m_compute=rows)
+    return time.perf_counter() - t0
+
+
+_GRID = {}
+
+
+def _scratch_grid(cfg):
+    if cfg.name not in _GRID:
+        _GRID[cfg.name] = np.zeros((cfg.dim, cfg.dim), np.int32)
+    return _GRID[cfg.name]
+
+
+def cpu_baseline(cfg, inputs, budget_s=12.0):
+    """The oracle as it stands, 1 thread, on a bounded row-prefix sample (~budget_s of work)."""
+    calib_rows = max(1, min(cfg.dim, 16))
+    t = oracle_sample(cfg, inputs, calib_rows)
+    per_row = max(t / calib_rows, 1e-7)
+    rows = int(max(calib_rows, min(cfg.dim, budget_s / per_row)))
+    reps = 1
+    t = oracle_sample(cfg, inputs, rows)
+    while rows == cfg.dim and t * (reps + 1) / reps < budget_s and reps < 5:
+        t += oracle_sample(cfg, inputs, rows)
+        reps += 1
+    cells = rows * cfg.dim * reps
+    return {"value": cells / t / 1e9, "unit": UNIT, "cores": 1, "kind": "oracle",
+            "sample": f"rows 1..{rows} x {cfg.dim} cols ({'full grid' if rows == cfg.dim else 'exact row prefix'})"
+                      f", {reps} run(s), {t:.1f} s single-thread"}
+
+
+def run_reference(args, cfg):
+    rank = _env_int("RANK", 0)
+    if rank != 0:
+        return 0
+    inputs = host_inputs(cfg)
+    calib = max(1, min(cfg.dim, 16))
+    per_row = oracle_sample(cfg, inputs, calib) / calib
+    budget = 120.0 / max(1, args.steps + args.warmup)
+    rows = int(max(1, min(cfg.dim, budget / max(per_row, 1e-9))))
+    for _ in range(args.warmup):
+        oracle_sample(cfg, inputs, rows)
+    times = [oracle_sample(cfg, inputs, rows) for _ in range(args.steps)]
+    tot = sum(times)
+    value = rows * cfg.dim * args.steps / tot / 1e9
+    line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": tot / args.steps * 1e3, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": dtype_of(cfg), "data": "synthetic",
+            "impl": "reference",
+            "config": {"workload": cfg.name + ": " + cfg.note, "fn": cfg.fn, "dim": cfg.dim, "tsize": cfg.tsize,
+                       "dsize": cfg.dsize, "sample_rows": rows},
+            "cpu_baseline": {"value": value, "unit": UNIT, "cores": 1, "kind": "oracle",
+                             "sample": f"each step: rows 1..{rows} x {cfg.dim} cols (exact row prefix)"},
+            "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line))
+    return 0
+
+
+def dtype_of(cfg):
+    return {"seqcmp": "int32", "synthetic": "int32+f32", "nash": "int32"}[cfg.fn]
+
+
+# ------------------------------------------------------------------------------------ our arm
+def run_ours(args, cfg):
+    import torch
+    import torch.distributed as dist
+
+    from paper_conf_ppopp_mohantyc14_b200.wf import Wavefront
+
+    world = _env_int("WORLD_SIZE", 1)
+    rank = _env_int("RANK", 0)
+    local = _env_int("LOCAL_RANK", 0)
+    if world != args.gpus:
+        raise SystemExit(f"--gpus {args.gpus} but WORLD_SIZE={world} (launch N>1 with torchrun)")
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if world > 1:
+        os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+        dist.init_process_group("nccl", device_id=dev)
+
+    tun = {}
+    for k in ("lane_cols", "warps", "skew"):
+        v = getattr(args, k)
+        if v:
+            tun[k] = v
+    w = Wavefront(cfg.fn, cfg.dim, rank=rank, device=local, ngpus=world, **fn_kwargs(cfg), **tun)
+    lay = w.layout
+    if world > 1:
+        handles = [None] * world
+        dist.all_gather_object(handles, w.ipc_handle())
+        w.connect(handles[rank - 1] if rank > 0 else None, handles[rank + 1] if rank < world - 1 else None)
+
+    inputs = host_inputs(cfg)
+    if cfg.fn == "seqcmp":
+        host = list(inputs)
+        tops, lefts = [], []
+    else:
+        row, col, top, left = inputs
+        host = [row, col]
+        tops = [torch.from_numpy(np.ascontiguousarray(top[p])).to(dev) for p in range(top.shape[0])]
+        lefts = [torch.from_numpy(np.ascontiguousarray(left[p])).to(dev) for p in range(left.shape[0])]
+    pinned = [torch.from_numpy(np.ascontiguousarray(a)).pin_memory() for a in host]
+    row_in, col_in = [p.to(dev) for p in pinned]
+    out = w.alloc_out()
+    stream = torch.cuda.current_stream()
+    slab_cells = cfg.dim * lay.width
+    total_cells = cfg.dim * cfg.dim
+    footprint = lay.bytes_out
+    flush = footprint < 2 * L2_BYTES
+    flush_buf = torch.empty(2 * L2_BYTES // 4, dtype=torch.int32, device=dev) if flush else None
+
+    def barrier():
+        if world > 1:
+            dist.barrier(device_ids=[local])
+        torch.cuda.synchronize()
+
+    for _ in range(args.warmup):
+        w.run(row_in, col_in, tops, lefts, out=out, stream=stream)
+    barrier()
+    w.sync()
+
+    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
+    t_start, t_end = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    with ClockSampler(local) as clk:
+        barrier()
+        t_start.record(stream)
+        for i in range(args.steps):
+            if flush:
+                flush_buf.fill_(i)
+            ev[i][0].record(stream)
+            w.run(row_in, col_in, tops, lefts, out=out, stream=stream)
+            ev[i][1].record(stream)
+        t_end.record(stream)
+        torch.cuda.synchronize()
+        barrier()
+    w.sync()
+    launch_ms = [a.elapsed_time(b) for a, b in ev]
+    step_ms_local = (sum(launch_ms) if flush else t_start.elapsed_time(t_end)) / args.steps
+    avg_launch_ms = sum(launch_ms) / len(launch_ms)
+    if world > 1:
+        tt = torch.tensor([step_ms_local], device=dev, dtype=torch.float64)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        step_ms = float(tt.item())
+    else:
+        step_ms = step_ms_local
+    value = total_cells / (step_ms * 1e-3) / 1e9
+
+    # ---- end to end through the public API: H2D inputs (pinned), sweep, D2H of the result
+    # (the last row of this slab = the alignment scores against every prefix of y)
+    e2e_steps = max(3, min(args.steps, 50))
+    res_host = torch.empty((lay.nplanes, lay.width), dtype=torch.int32).pin_memory()
+    barrier()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(e2e_steps):
+        r_d = pinned[0].to(dev, non_blocking=True)
+        c_d = pinned[1].to(dev, non_blocking=True)
+        o = w.run(r_d, c_d, tops, lefts, out=out, stream=stream)
+        for f in range(lay.nplanes):
+            res_host[f].copy_(o[f][-1].view(torch.int32), non_blocking=True)
+    e1.record(stream)
+    torch.cuda.synchronize()
+    w.sync()
+    e2e_ms = e0.elapsed_time(e1) / e2e_steps
+    if world > 1:
+        tt = torch.tensor([e2e_ms], device=dev, dtype=torch.float64)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        e2e_ms = float(tt.item())
+    h2d = sum(p.numel() * p.element_size() for p in pinned)
+    d2h = res_host.numel() * res_host.element_size()
+
+    # ---- full-grid variant (the paper timed the whole program incl. the result copy-back)
+    grid_e2e = None
+    if args.e2e_grid and world == 1:
+        host_grid = [torch.empty((cfg.dim, lay.width), dtype=o_.dtype).pin_memory() for o_ in out]
+        torch.cuda.synchronize()
+        g0, g1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        reps = 2
+        g0.record(stream)
+        for _ in range(reps):
+            r_d = pinned[0].to(dev, non_blocking=True)
+            c_d = pinned[1].to(dev, non_blocking=True)
+            o = w.run(r_d, c_d, tops, lefts, out=out, stream=stream)
+            for f in range(lay.nplanes):
+                host_grid[f].copy_(o[f], non_blocking=True)
+        g1.record(stream)
+        torch.cuda.synchronize()
+        gms = g0.elapsed_time(g1) / reps
+        grid_e2e = {"value": total_cells / (gms * 1e-3) / 1e9, "unit": UNIT, "ms_per_step": gms,
+                    "d2h_bytes_per_step": int(footprint), "h2d_bytes_per_step": h2d}
+        del host_grid
+
+    peak, peak_src = load_peaks()
+    bytes_per_launch = slab_cells * cfg.bytes_per_cell()
+    achieved = bytes_per_launch / (avg_launch_ms * 1e-3) / 1e9
+    key = f"{cfg.name}_k{lay.lane_cols}w{lay.warps}d{lay.skew}"
+    traffic = load_traffic(key)
+
+    result = None
+    if rank == 0:
+        result = {
+            "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": step_ms, "higher_is_better": True, "scaling": "weak" if False else "strong",
+            "vs_baseline": None, "dtype": dtype_of(cfg), "data": "synthetic (seeded PCG64 inputs, workloads/)",
+            "config": {"workload": cfg.name + ": " + cfg.note, "fn": cfg.fn, "dim": cfg.dim, "tsize": cfg.tsize,
+                       "dsize": cfg.dsize, "lane_cols": lay.lane_cols, "warps": lay.warps, "skew": lay.skew,
+                       "band_cols": lay.band_cols, "nbands_per_slab": lay.nbands,
+                       "parallelism": f"column slabs x{world}" if world > 1 else "1 GPU",
+                       "l2": ("explicit 252 MiB L2 flush between steps (footprint < 2x L2)" if flush else
+                              f"outputs {footprint / 2**30:.2f} GiB per GPU > 126 MB L2; no flush needed")},
+            "gpu_launches": args.steps * world,
+            "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
+                         "traffic": traffic, "peak_source": peak_src,
+                         "algorithmic_bytes_per_launch": bytes_per_launch, "avg_launch_ms": avg_launch_ms,
+                         "kernel": "wfk::sweep_kernel"},
+            "e2e": {"value": total_cells / (e2e_ms * 1e-3) / 1e9, "unit": UNIT, "ms_per_step": e2e_ms,
+                    "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
+                    "note": "H2D of the step's inputs from pinned memory, sweep, D2H of the result row"},
+            "clocks": clk.summary(),
+        }
+        if grid_e2e:
+            result["e2e_full_grid"] = grid_e2e
+    w.close()
+    if world > 1:
+        dist.barrier(device_ids=[local])
+        dist.destroy_process_group()
+    if rank == 0:
+        if world == 1 and not args.no_cpu_baseline:
+            result["cpu_baseline"] = cpu_baseline(cfg, inputs)
+            import multiprocessing
+            result["cpu_baseline"]["host_cpus"] = multiprocessing.cpu_count()
+        result["scaling"] = "strong"
+        print(json.dumps(result))
+    return 0
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=200)
+    ap.add_argument("--warmup", type=int, default=10)
+    ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
+    ap.add_argument("--config", default="C4", choices=sorted(workloads.CONFIGS))
+    ap.add_argument("--lane-cols", dest="lane_cols", type=int, default=0)
+    ap.add_argument("--warps", type=int, default=0)
+    ap.add_argument("--skew", type=int, default=0)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--e2e-grid", dest="e2e_grid", action="store_true", default=True)
+    ap.add_argument("--no-e2e-grid", dest="e2e_grid", action="store_false")
+    args = ap.parse_args()
+    if args.warmup < 3:
+        raise SystemExit("--warmup must be >= 3")
+    cfg = workloads.CONFIGS[args.config]
+    if args.impl == "reference":
+        return run_reference(args, cfg)
+    return run_ours(args, cfg)
+
+
+if __name__ == "__main__":
+    sys.exit(main())

@@ -1,0 +1,502 @@
+// wf_api.cpp -- the C ABI of libwf (include/wf.h): parameter validation, the planner
+// (bands, slabs, persistent grid), library-owned scratch, and the launch path.
+//
+// The planner replaces the paper's tunables (Table 2: cpu-tile, band,
+// gpu-count, gpu-tile, halo) with the B200 sweep's: lane columns k, warps per CTA band,
+// lane skew d, GPU (slab) count and transport (DESIGN.md §6 "what differs from the paper").
+#include <cuda_runtime.h>
+
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <new>
+#include <string>
+
+#include "../../include/wf.h"
+#include "wf_internal.h"
+
+namespace wfk {
+int variant_count();
+}
+
+struct wf_ctx {
+  wf_params p{};
+  int rank = 0, world = 1, device = 0, share = 1;
+  int nf = 1, nbound = 0;
+  int c0 = 0, c1 = 0;
+  int k = 4, warps = 2, skew = 2, band_w = 256, nbands = 1;
+  int grid = 1;
+  int smem = 0;
+  void* base = nullptr;                    // one allocation: [control block | edge rings] (IPC-exportable)
+  unsigned* ack = nullptr;                 // control word written by the successor slab
+  unsigned long long* edge = nullptr;      // nbands * rows * nf LL words (library-owned)
+  size_t edge_bytes = 0;
+  unsigned* ack_prev = nullptr;            // predecessor's control word (local / peer / IPC)
+  void* prev_ipc_base = nullptr;
+  unsigned long long* next_edge = nullptr; // next slab's band-0 ring (peer / IPC / local)
+  void* next_ipc_base = nullptr;
+  int* err = nullptr;                      // device error word
+  uint32_t epoch = 0;
+  cudaEvent_t ev0 = nullptr, ev1 = nullptr;
+  bool ran = false;
+  std::string msg;
+};
+
+namespace {
+
+thread_local std::string g_last_error;
+constexpr size_t kCtrlBytes = 256;   // control block at the head of the IPC-exportable allocation
+
+wf_status fail(wf_ctx* c, wf_status st, const char* fmt, ...) {
+  char buf[512];
+  va_list ap;
+  va_start(ap, fmt);
+  vsnprintf(buf, sizeof buf, fmt, ap);
+  va_end(ap);
+  if (c) c->msg = buf;
+  else g_last_error = buf;
+  return st;
+}
+
+wf_status cuda_fail(wf_ctx* c, cudaError_t e, const char* what) {
+  cudaGetLastError();
+  return fail(c, e == cudaErrorMemoryAllocation ? WF_ENOMEM : WF_ECUDA, "%s: %s", what, cudaGetErrorString(e));
+}
+
+struct Plan {
+  int nf, nbound, k, warps, skew, band_w, c0, c1, nbands;
+  int match, mismatch, gap;
+};
+
+// Defaults until the autotune table says otherwise (tools/autotune.py).
+void defaults(const wf_params& p, int* k, int* w, int* d) {
+  if (p.fn == WF_FN_SEQCMP) {
+    *k = p.lane_cols ? p.lane_cols : 4;
+    *w = p.warps ? p.warps : 2;
+    *d = p.skew ? p.skew : 2;
+  } else {
+    *k = p.lane_cols ? p.lane_cols : 1;
+    *w = p.warps ? p.warps : 2;
+    *d = p.skew ? p.skew : 1;
+  }
+}
+
+wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
+  if (!p) return fail(c, WF_EINVAL, "params is NULL");
+  const int rows = p->dim;
+  const int cols = p->cols ? p->cols : p->dim;
+  if (rows < 1 || rows > 65535) return fail(c, WF_EINVAL, "dim=%d out of range 1..65535", rows);
+  if (cols < 1 || cols > 65535) return fail(c, WF_EINVAL, "cols=%d out of range 1..65535", cols);
+  for (int i = 0; i < 6; ++i)
+    if (p->reserved[i]) return fail(c, WF_EINVAL, "reserved[%d] must be 0", i);
+  if (p->ngpus < 0 || p->ngpus > 8) return fail(c, WF_EINVAL, "ngpus=%d out of range 1..8", p->ngpus);
+  const int G = p->ngpus ? p->ngpus : 1;
+  if (rank < 0 || rank >= G) return fail(c, WF_EINVAL, "rank=%d out of range for ngpus=%d", rank, G);
+  if (p->transport > WF_TRANSPORT_NCCL) return fail(c, WF_EINVAL, "transport=%u unknown", p->transport);
+  if (p->strip < 0) return fail(c, WF_EINVAL, "strip=%d must be >= 0", p->strip);
+  if (p->lane_cols < 0 || p->warps < 0 || p->skew < 0)
+    return fail(c, WF_EINVAL, "lane_cols/warps/skew must be >= 0");
+  Plan pl{};
+  switch (p->fn) {
+    case WF_FN_SEQCMP: {
+      if (p->tsize != 0) return fail(c, WF_EINVAL, "tsize=%d must be 0 for SEQCMP", p->tsize);
+      if (p->dsize != 0) return fail(c, WF_EINVAL, "dsize=%d must be 0 for SEQCMP", p->dsize);
+      if (p->local != 0 && p->local != 1) return fail(c, WF_EINVAL, "local=%d must be 0 or 1", p->local);
+      if (p->local == 1) return fail(c, WF_EUNSUPPORTED, "local=1 (Smith-Waterman) is not built in ABI v1");
+      const bool def = p->match == 0 && p->mismatch == 0 && p->gap == 0;
+      pl.match = def ? 1 : p->match;
+      pl.mismatch = def ? -1 : p->mismatch;
+      pl.gap = def ? -1 : p->gap;
+      if (pl.match < -64 || pl.match > 64) return fail(c, WF_EINVAL, "match=%d out of [-64,64]", pl.match);
+      if (pl.mismatch < -64 || pl.mismatch > 64) return fail(c, WF_EINVAL, "mismatch=%d out of [-64,64]", pl.mismatch);
+      if (pl.gap < -64 || pl.gap > 64) return fail(c, WF_EINVAL, "gap=%d out of [-64,64]", pl.gap);
+      pl.nf = 1;
+      pl.nbound = 0;
+      break;
+    }
+    case WF_FN_SYNTHETIC:
+      if (p->tsize < 0 || p->tsize > 1000000) return fail(c, WF_EINVAL, "tsize=%d out of range 0..1000000", p->tsize);
+      if (p->dsize < 0 || p->dsize > 8) return fail(c, WF_EINVAL, "dsize=%d out of range 0..8", p->dsize);
+      if ((long long)rows * cols > 2147483647LL && rows > 46340)
+        return fail(c, WF_EINVAL, "dim too large for the int32 i1 = i*j field");
+      pl.nf = 2 + p->dsize;
+      pl.nbound = p->dsize;
+      break;
+    case WF_FN_NASH:
+      if (p->tsize < 1 || p->tsize > 64) return fail(c, WF_EINVAL, "tsize=%d (strategies) out of range 1..64", p->tsize);
+      if (p->dsize != 4) return fail(c, WF_EINVAL, "dsize=%d must be 4 for NASH", p->dsize);
+      return fail(c, WF_EUNSUPPORTED, "fn=NASH kernel not built yet");
+    default:
+      return fail(c, WF_EINVAL, "fn=%d unknown", p->fn);
+  }
+  defaults(*p, &pl.k, &pl.warps, &pl.skew);
+  if (pl.k != 1 && pl.k != 2 && pl.k != 4 && pl.k != 8) return fail(c, WF_EINVAL, "lane_cols=%d not in {1,2,4,8}", pl.k);
+  if (pl.warps < 1 || pl.warps > 8) return fail(c, WF_EINVAL, "warps=%d out of range 1..8", pl.warps);
+  if (pl.skew < 1 || pl.skew > 4) return fail(c, WF_EINVAL, "skew=%d out of range 1..4", pl.skew);
+  if (!wfk::variant_exists(p->fn, p->dsize, pl.k, pl.warps, pl.skew))
+    return fail(c, WF_EUNSUPPORTED, "no kernel variant for fn=%d dsize=%d lane_cols=%d warps=%d skew=%d", p->fn,
+                p->dsize, pl.k, pl.warps, pl.skew);
+  pl.band_w = pl.warps * 32 * pl.k;
+  // slabs: every slab but the last is a whole number of bands (its east column is then
+  // owned by the last lane of its last band); bands are dealt out as evenly as possible
+  const long long B = (cols + pl.band_w - 1) / pl.band_w;
+  const long long b0 = B * rank / G, b1 = B * (rank + 1) / G;
+  pl.c0 = (int)(b0 * pl.band_w < cols ? b0 * pl.band_w : cols);
+  pl.c1 = (int)(b1 * pl.band_w < cols ? b1 * pl.band_w : cols);
+  if (pl.c1 <= pl.c0) return fail(c, WF_EINVAL, "ngpus=%d leaves slab %d empty (cols=%d, band=%d)", G, rank, cols, pl.band_w);
+  pl.nbands = (pl.c1 - pl.c0 + pl.band_w - 1) / pl.band_w;
+  *out = pl;
+  return WF_OK;
+}
+
+}  // namespace
+
+extern "C" {
+
+int32_t wf_abi_version(void) { return WF_ABI_VERSION; }
+
+const char* wf_build_info(void) {
+  static std::string s;
+  if (s.empty()) {
+    char b[256];
+    snprintf(b, sizeof b, "libwf abi=%d arch=sm_100a variants=%d cuda=%d", WF_ABI_VERSION, wfk::variant_count(),
+             CUDART_VERSION);
+    s = b;
+  }
+  return s.c_str();
+}
+
+const char* wf_last_error(const wf_ctx* c) {
+  if (c) return c->msg.c_str();
+  return g_last_error.c_str();
+}
+
+wf_status wf_query(const wf_params* p, int32_t rank, wf_layout* out) {
+  if (!out) return fail(nullptr, WF_EINVAL, "layout is NULL");
+  Plan pl;
+  wf_status st = validate(p, rank, &pl, nullptr);
+  if (st != WF_OK) return st;
+  memset(out, 0, sizeof *out);
+  out->nplanes = pl.nf;
+  for (int f = 0; f < pl.nf; ++f) {
+    out->plane_bytes[f] = 4;
+    out->plane_is_float[f] = (p->fn == WF_FN_SYNTHETIC && f >= 2) ? 1 : 0;
+  }
+  out->nbound = pl.nbound;
+  out->col_begin = pl.c0;
+  out->col_end = pl.c1;
+  out->min_pitch = ((int64_t)(pl.c1 - pl.c0) + 3) / 4 * 4;
+  out->bytes_out = out->min_pitch * p->dim * 4 * pl.nf;
+  out->lane_cols = pl.k;
+  out->warps = pl.warps;
+  out->skew = pl.skew;
+  out->band_cols = pl.band_w;
+  out->nbands = pl.nbands;
+  return WF_OK;
+}
+
+wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
+  if (!out) return fail(nullptr, WF_EINVAL, "out is NULL");
+  *out = nullptr;
+  const int rank = dist ? dist->rank : 0;
+  if (dist) {
+    const int G = p && p->ngpus ? p->ngpus : 1;
+    if (dist->world != G) return fail(nullptr, WF_EINVAL, "dist.world=%d != params.ngpus=%d", dist->world, G);
+    if (dist->device_share < 0 || dist->device_share > 64)
+      return fail(nullptr, WF_EINVAL, "dist.device_share=%d out of range", dist->device_share);
+  } else if (p && p->ngpus > 1) {
+    return fail(nullptr, WF_EINVAL, "ngpus=%d needs a wf_dist", p->ngpus);
+  }
+  Plan pl;
+  wf_status st = validate(p, rank, &pl, nullptr);
+  if (st != WF_OK) return st;
+
+  wf_ctx* c = new (std::nothrow) wf_ctx();
+  if (!c) return fail(nullptr, WF_ENOMEM, "host allocation failed");
+  c->p = *p;
+  c->rank = rank;
+  c->world = dist ? dist->world : 1;
+  c->share = dist && dist->device_share > 1 ? dist->device_share : 1;
+  c->nf = pl.nf;
+  c->nbound = pl.nbound;
+  c->c0 = pl.c0;
+  c->c1 = pl.c1;
+  c->k = pl.k;
+  c->warps = pl.warps;
+  c->skew = pl.skew;
+  c->band_w = pl.band_w;
+  c->nbands = pl.nbands;
+  c->p.match = pl.match;
+  c->p.mismatch = pl.mismatch;
+  c->p.gap = pl.gap;
+
+  cudaError_t e;
+  if (dist && dist->device >= 0) {
+    e = cudaSetDevice(dist->device);
+    if (e != cudaSuccess) {
+      st = cuda_fail(nullptr, e, "cudaSetDevice");
+      delete c;
+      return st;
+    }
+  }
+  e = cudaGetDevice(&c->device);
+  if (e != cudaSuccess) {
+    st = cuda_fail(nullptr, e, "cudaGetDevice");
+    delete c;
+    return st;
+  }
+  // persistent grid: every CTA must be co-resident (flags are spun on, never relaunched)
+  wfk::SweepLaunch L{};
+  L.fn = p->fn;
+  L.dsize = p->dsize;
+  L.k = pl.k;
+  L.warps = pl.warps;
+  L.skew = pl.skew;
+  c->smem = wfk::smem_bytes(L);
+  int sms = 0, optin = 0;
+  cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, c->device);
+  cudaDeviceGetAttribute(&optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, c->device);
+  if (c->smem < 0 || c->smem > optin) {
+    fail(nullptr, WF_EUNSUPPORTED, "variant needs %d B shared memory (device max %d)", c->smem, optin);
+    delete c;
+    return WF_EUNSUPPORTED;
+  }
+  const int occ = wfk::occupancy(L, c->smem);
+  if (occ < 1) {
+    fail(nullptr, WF_EUNSUPPORTED, "kernel variant cannot be resident (occupancy 0)");
+    delete c;
+    return WF_EUNSUPPORTED;
+  }
+  int cap = occ * sms / c->share;
+  if (cap < 1) cap = 1;
+  c->grid = pl.nbands < cap ? pl.nbands : cap;
+  if (p->max_ctas && (int)p->max_ctas < c->grid) c->grid = (int)p->max_ctas;
+  if (c->grid < 1) c->grid = 1;
+
+  c->edge_bytes = (size_t)pl.nbands * p->dim * pl.nf * sizeof(unsigned long long);
+  e = cudaMalloc(&c->base, kCtrlBytes + c->edge_bytes);
+  if (e == cudaSuccess) e = cudaMemset(c->base, 0, kCtrlBytes + c->edge_bytes);
+  if (e == cudaSuccess) {
+    c->ack = static_cast<unsigned*>(c->base);
+    c->edge = reinterpret_cast<unsigned long long*>(static_cast<char*>(c->base) + kCtrlBytes);
+  }
+  if (e == cudaSuccess) e = cudaMalloc(&c->err, sizeof(int));
+  if (e == cudaSuccess) e = cudaMemset(c->err, 0, sizeof(int));
+  if (e == cudaSuccess) e = cudaEventCreate(&c->ev0);
+  if (e == cudaSuccess) e = cudaEventCreate(&c->ev1);
+  if (e == cudaSuccess) e = cudaDeviceSynchronize();
+  if (e != cudaSuccess) {
+    st = cuda_fail(nullptr, e, "wf_create scratch");
+    wf_destroy(c);
+    return st;
+  }
+  *out = c;
+  return WF_OK;
+}
+
+wf_status wf_destroy(wf_ctx* c) {
+  if (!c) return WF_OK;
+  int prev = -1;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  if (c->ev1) cudaEventSynchronize(c->ev1);
+  if (c->next_ipc_base) cudaIpcCloseMemHandle(c->next_ipc_base);
+  if (c->prev_ipc_base) cudaIpcCloseMemHandle(c->prev_ipc_base);
+  if (c->base) cudaFree(c->base);
+  if (c->err) cudaFree(c->err);
+  if (c->ev0) cudaEventDestroy(c->ev0);
+  if (c->ev1) cudaEventDestroy(c->ev1);
+  if (prev >= 0) cudaSetDevice(prev);
+  cudaGetLastError();
+  delete c;
+  return WF_OK;
+}
+
+wf_status wf_link_local(wf_ctx* prev, wf_ctx* next) {
+  if (!prev || !next) return fail(prev, WF_EINVAL, "wf_link_local: NULL context");
+  if (next->rank != prev->rank + 1 || next->world != prev->world)
+    return fail(prev, WF_EINVAL, "wf_link_local: ranks %d -> %d are not consecutive slabs", prev->rank, next->rank);
+  if (prev->nf != next->nf || prev->p.dim != next->p.dim)
+    return fail(prev, WF_EINVAL, "wf_link_local: contexts describe different problems");
+  if (prev->device != next->device) {
+    int can = 0;
+    cudaDeviceCanAccessPeer(&can, prev->device, next->device);
+    if (!can) return fail(prev, WF_ECOMM, "device %d cannot access peer %d", prev->device, next->device);
+    int cur = 0;
+    cudaGetDevice(&cur);
+    cudaSetDevice(prev->device);
+    cudaError_t e = cudaDeviceEnablePeerAccess(next->device, 0);
+    cudaSetDevice(cur);
+    if (e != cudaSuccess && e != cudaErrorPeerAccessAlreadyEnabled) {
+      cudaGetLastError();
+      return fail(prev, WF_ECOMM, "cudaDeviceEnablePeerAccess(%d->%d): %s", prev->device, next->device,
+                  cudaGetErrorString(e));
+    }
+    cudaGetLastError();
+  }
+  if (next->device != prev->device) {
+    int cur = 0;
+    cudaGetDevice(&cur);
+    cudaSetDevice(next->device);
+    cudaError_t e = cudaDeviceEnablePeerAccess(prev->device, 0);   // next writes prev's ack word
+    cudaSetDevice(cur);
+    if (e != cudaSuccess && e != cudaErrorPeerAccessAlreadyEnabled) {
+      cudaGetLastError();
+      return fail(prev, WF_ECOMM, "cudaDeviceEnablePeerAccess(%d->%d): %s", next->device, prev->device,
+                  cudaGetErrorString(e));
+    }
+    cudaGetLastError();
+  }
+  prev->next_edge = next->edge;   // next slab's band-0 inbound ring
+  next->ack_prev = prev->ack;     // next acknowledges each drained run into prev's control word
+  return WF_OK;
+}
+
+wf_status wf_ipc_handle(wf_ctx* c, void* handle) {
+  if (!c || !handle) return fail(c, WF_EINVAL, "wf_ipc_handle: NULL argument");
+  cudaIpcMemHandle_t h;
+  cudaError_t e = cudaIpcGetMemHandle(&h, c->base);
+  if (e != cudaSuccess) {
+    cudaGetLastError();
+    return fail(c, WF_ECOMM, "cudaIpcGetMemHandle: %s", cudaGetErrorString(e));
+  }
+  static_assert(sizeof(h) == WF_IPC_HANDLE_BYTES, "IPC handle size");
+  memcpy(handle, &h, sizeof h);
+  return WF_OK;
+}
+
+static wf_status open_ipc(wf_ctx* c, const void* handle, void** out) {
+  cudaIpcMemHandle_t h;
+  memcpy(&h, handle, sizeof h);
+  cudaError_t e = cudaIpcOpenMemHandle(out, h, cudaIpcMemLazyEnablePeerAccess);
+  if (e != cudaSuccess) {
+    cudaGetLastError();
+    return fail(c, WF_ECOMM, "cudaIpcOpenMemHandle: %s", cudaGetErrorString(e));
+  }
+  return WF_OK;
+}
+
+wf_status wf_connect(wf_ctx* c, const void* prev_handle, const void* next_handle) {
+  if (!c) return fail(c, WF_EINVAL, "wf_connect: NULL context");
+  if ((c->rank > 0) != (prev_handle != nullptr))
+    return fail(c, WF_EINVAL, "wf_connect: rank %d %s a predecessor handle", c->rank, c->rank > 0 ? "needs" : "takes no");
+  if ((c->rank < c->world - 1) != (next_handle != nullptr))
+    return fail(c, WF_EINVAL, "wf_connect: rank %d %s a successor handle", c->rank,
+                c->rank < c->world - 1 ? "needs" : "takes no");
+  int cur = 0;
+  cudaGetDevice(&cur);
+  cudaSetDevice(c->device);
+  wf_status st = WF_OK;
+  if (next_handle) {
+    void* p = nullptr;
+    st = open_ipc(c, next_handle, &p);
+    if (st == WF_OK) {
+      c->next_ipc_base = p;
+      c->next_edge = reinterpret_cast<unsigned long long*>(static_cast<char*>(p) + kCtrlBytes);
+    }
+  }
+  if (st == WF_OK && prev_handle) {
+    void* p = nullptr;
+    st = open_ipc(c, prev_handle, &p);
+    if (st == WF_OK) {
+      c->prev_ipc_base = p;
+      c->ack_prev = static_cast<unsigned*>(p);
+    }
+  }
+  cudaSetDevice(cur);
+  return st;
+}
+
+wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
+  if (!c) return fail(nullptr, WF_EINVAL, "wf_run: NULL context");
+  if (!io) return fail(c, WF_EINVAL, "wf_run: io is NULL");
+  const wf_params& p = c->p;
+  const int cols = p.cols ? p.cols : p.dim;
+  if (c->world > 1 && c->rank < c->world - 1 && !c->next_edge)
+    return fail(c, WF_ESTATE, "wf_run: slab %d is not linked to its successor (wf_link_local / wf_connect)", c->rank);
+  if (!io->row_in || !io->col_in) return fail(c, WF_EINVAL, "wf_run: row_in/col_in must be device pointers");
+  const int64_t min_pitch = ((int64_t)(c->c1 - c->c0) + 3) / 4 * 4;
+  if (io->out_pitch < min_pitch || io->out_pitch % 4 != 0)
+    return fail(c, WF_EINVAL, "wf_run: out_pitch=%lld must be a multiple of 4 and >= %lld", (long long)io->out_pitch,
+                (long long)min_pitch);
+  for (int f = 0; f < c->nf; ++f) {
+    if (!io->out[f]) return fail(c, WF_EINVAL, "wf_run: out[%d] is NULL", f);
+    if (reinterpret_cast<uintptr_t>(io->out[f]) % 16) return fail(c, WF_EINVAL, "wf_run: out[%d] not 16-byte aligned", f);
+  }
+  for (int b = 0; b < c->nbound; ++b)
+    if (!io->top[b] || !io->left[b]) return fail(c, WF_EINVAL, "wf_run: top[%d]/left[%d] must be set", b, b);
+
+  wfk::SweepLaunch L{};
+  L.fn = p.fn;
+  L.rows = p.dim;
+  L.cols = cols;
+  L.tsize = p.tsize;
+  L.dsize = p.dsize;
+  L.c0 = c->c0;
+  L.c1 = c->c1;
+  L.match = p.match;
+  L.mismatch = p.mismatch;
+  L.gap = p.gap;
+  L.k = c->k;
+  L.warps = c->warps;
+  L.skew = c->skew;
+  L.band_w = c->band_w;
+  L.nbands = c->nbands;
+  L.grid = c->grid;
+  L.row_in = io->row_in;
+  L.col_in = io->col_in;
+  for (int f = 0; f < WF_MAX_PLANES; ++f) {
+    L.top[f] = io->top[f];
+    L.left[f] = io->left[f];
+    L.out[f] = io->out[f];
+  }
+  L.pitch = io->out_pitch;
+  L.edge = c->edge;
+  L.next_edge = c->next_edge;
+  L.ack_self = c->ack;
+  L.ack_prev = c->ack_prev;
+  L.first_slab = c->rank == 0;
+  L.epoch = ++c->epoch;
+  if ((L.epoch & 0x0FFFFFFFu) == 0) L.epoch = ++c->epoch;   // tag 0 marks "never written"
+  L.err = c->err;
+  L.watchdog = p.watchdog_cycles ? p.watchdog_cycles : (1ull << 32);
+
+  int prev = -1;
+  cudaGetDevice(&prev);
+  if (prev != c->device) cudaSetDevice(c->device);
+  cudaStream_t s = static_cast<cudaStream_t>(cuda_stream);
+  cudaError_t e = cudaEventRecord(c->ev0, s);
+  if (e == cudaSuccess) e = wfk::launch(L, s);
+  if (e == cudaSuccess) e = cudaEventRecord(c->ev1, s);
+  if (prev >= 0 && prev != c->device) cudaSetDevice(prev);
+  if (e != cudaSuccess) return cuda_fail(c, e, "wf_run launch");
+  c->ran = true;
+  return WF_OK;
+}
+
+wf_status wf_sync(wf_ctx* c) {
+  if (!c) return fail(nullptr, WF_EINVAL, "wf_sync: NULL context");
+  if (!c->ran) return WF_OK;
+  cudaError_t e = cudaEventSynchronize(c->ev1);
+  if (e != cudaSuccess) return cuda_fail(c, e, "wf_sync");
+  int w = 0;
+  e = cudaMemcpy(&w, c->err, sizeof w, cudaMemcpyDeviceToHost);
+  if (e != cudaSuccess) return cuda_fail(c, e, "wf_sync error word");
+  if (((unsigned)w >> 4) == (c->epoch & 0x0FFFFFFFu) && (w & 15) == wfk::DEV_TIMEOUT)
+    return fail(c, WF_ETIMEOUT, "watchdog: a dependency wait exceeded %llu cycles (run epoch %u)",
+                (unsigned long long)(c->p.watchdog_cycles ? c->p.watchdog_cycles : (1ull << 32)), c->epoch);
+  return WF_OK;
+}
+
+wf_status wf_last_run_ms(wf_ctx* c, float* ms) {
+  if (!c || !ms) return fail(c, WF_EINVAL, "wf_last_run_ms: NULL argument");
+  if (!c->ran) return fail(c, WF_ESTATE, "wf_last_run_ms: no run yet");
+  cudaError_t e = cudaEventQuery(c->ev1);
+  if (e == cudaErrorNotReady) return fail(c, WF_ESTATE, "wf_last_run_ms: run still in flight");
+  if (e != cudaSuccess) return cuda_fail(c, e, "wf_last_run_ms");
+  e = cudaEventElapsedTime(ms, c->ev0, c->ev1);
+  if (e != cudaSuccess) return cuda_fail(c, e, "cudaEventElapsedTime");
+  return WF_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,57 @@
+// wf_internal.h -- host-side launch interface between the C-ABI layer (wf_api.cpp)
+// and the sm_100a kernels (wf_sweep.cu).  Not part of the public ABI.
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+#include "../../include/wf.h"
+
+namespace wfk {
+
+// Everything one slab's persistent launch needs.
+struct SweepLaunch {
+  // problem
+  int32_t fn, rows, cols, tsize, dsize;
+  int32_t c0, c1;                 // slab interior columns [c0, c1), 0-based
+  int32_t match, mismatch, gap;
+  // tuning
+  int32_t k, warps, skew;         // lane columns, compute warps per CTA, lane skew
+  int32_t band_w, nbands;         // band_w = warps*32*k
+  int32_t grid;                   // persistent CTAs (all co-resident)
+  // io
+  const void* row_in;
+  const void* col_in;
+  const void* top[WF_MAX_PLANES];
+  const void* left[WF_MAX_PLANES];
+  void* out[WF_MAX_PLANES];
+  int64_t pitch;
+  // edges: edge[b] (b = 0..nbands-1) is band b's inbound LL ring, rows*nf u64 each.
+  // edge[0] of slab g > 0 is written by slab g-1 (possibly through a peer mapping).
+  unsigned long long* edge;
+  unsigned long long* next_edge;  // inbound ring of slab g+1's band 0 (NULL on the last slab)
+  // Cross-run back-pressure between slabs: slab g+1's band-0 feeder stores the epoch it has
+  // fully consumed into slab g's ack word (ack_prev, possibly a peer address); slab g waits
+  // for ack_self >= epoch-1 before its first store into next_edge.
+  unsigned* ack_self;
+  unsigned* ack_prev;
+  int32_t first_slab;             // 1: band 0's west input is the column-0 boundary
+  uint32_t epoch;
+  int* err;                       // device error word
+  unsigned long long watchdog;
+};
+
+// Words per cell (= output planes) for a function.
+int nwords(int fn, int dsize);
+// Dynamic shared memory the kernel variant needs; <0 if the variant is not compiled.
+int smem_bytes(const SweepLaunch& L);
+// Max co-resident CTAs per SM for the variant (0 if it cannot launch).
+int occupancy(const SweepLaunch& L, int smem);
+// Launch (asynchronous).  Returns cudaSuccess or the launch error.
+cudaError_t launch(const SweepLaunch& L, cudaStream_t s);
+// Is (fn, dsize, k, warps, skew) compiled?
+bool variant_exists(int fn, int dsize, int k, int warps, int skew);
+
+// Error word codes (device side).
+enum : int { DEV_OK = 0, DEV_TIMEOUT = 1 };
+
+}  // namespace wfk

@@ -1,0 +1,128 @@
+// wf_sweep.cu -- instantiations and host-side launch of the persistent band sweep.
+#include <cstdio>
+#include <cstring>
+#include <type_traits>
+
+#include "wf_cells.cuh"
+#include "wf_sweep.cuh"
+
+namespace wfk {
+
+int nwords(int fn, int dsize) {
+  switch (fn) {
+    case WF_FN_SEQCMP: return 1;
+    case WF_FN_SYNTHETIC: return 2 + dsize;
+    case WF_FN_NASH: return 4;
+    default: return 0;
+  }
+}
+
+namespace {
+
+struct Variant {
+  int fn, dsize, k, warps, skew;
+  size_t smem;
+  const void* kernel;  // __global__ function pointer (for occupancy queries)
+  cudaError_t (*launch)(const SweepLaunch&, cudaStream_t, size_t);
+};
+
+template <class P, int K, int W, int D>
+cudaError_t launch_t(const SweepLaunch& L, cudaStream_t s, size_t smem) {
+  P pol{};
+  if constexpr (std::is_same<P, PolSeq>::value) {
+    pol.x = static_cast<const uint8_t*>(L.row_in);
+    pol.y = static_cast<const uint8_t*>(L.col_in);
+    pol.match = L.match;
+    pol.mismatch = L.mismatch;
+    pol.gap = L.gap;
+  } else {
+    pol.u = static_cast<const float*>(L.row_in);
+    pol.v = static_cast<const float*>(L.col_in);
+    for (int d = 0; d < L.dsize && d < (int)(sizeof(pol.topf) / sizeof(pol.topf[0])); ++d) {
+      pol.topf[d] = static_cast<const float*>(L.top[d]);
+      pol.leftf[d] = static_cast<const float*>(L.left[d]);
+    }
+    pol.tsize = L.tsize;
+  }
+  auto kfn = sweep_kernel<P, K, W, D>;
+  cudaError_t e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  if (e != cudaSuccess) return e;
+  kfn<<<L.grid, (W + 1) * 32, smem, s>>>(L, pol);
+  return cudaGetLastError();
+}
+
+template <class P, int K, int W, int D>
+Variant make_variant(int fn, int dsize) {
+  using S = Smem<P::NF, K, W, D>;
+  return Variant{fn, dsize, K, W, D, S::bytes, reinterpret_cast<const void*>(sweep_kernel<P, K, W, D>),
+                 &launch_t<P, K, W, D>};
+}
+
+// --- the compiled variant set -------------------------------------------------------
+#define WF_SEQ(K, W, D) make_variant<PolSeq, K, W, D>(WF_FN_SEQCMP, 0)
+#define WF_SYN(DS, K, W, D) make_variant<PolSyn<DS>, K, W, D>(WF_FN_SYNTHETIC, DS)
+#define WF_SYN_DS(DS) WF_SYN(DS, 1, 1, 1), WF_SYN(DS, 1, 2, 1), WF_SYN(DS, 1, 4, 1), WF_SYN(DS, 2, 1, 1), \
+    WF_SYN(DS, 2, 2, 1), WF_SYN(DS, 1, 2, 2), WF_SYN(DS, 2, 2, 2)
+
+const Variant* table(size_t* n) {
+  static const Variant v[] = {
+      WF_SEQ(2, 1, 1), WF_SEQ(2, 2, 1), WF_SEQ(2, 4, 1), WF_SEQ(2, 1, 2), WF_SEQ(2, 2, 2), WF_SEQ(2, 4, 2),
+      WF_SEQ(2, 2, 3), WF_SEQ(2, 4, 3),
+      WF_SEQ(4, 1, 1), WF_SEQ(4, 2, 1), WF_SEQ(4, 4, 1), WF_SEQ(4, 1, 2), WF_SEQ(4, 2, 2), WF_SEQ(4, 4, 2),
+      WF_SEQ(4, 1, 3), WF_SEQ(4, 2, 3), WF_SEQ(4, 4, 3),
+      WF_SEQ(8, 1, 1), WF_SEQ(8, 2, 1), WF_SEQ(8, 1, 2), WF_SEQ(8, 2, 2),
+      WF_SEQ(1, 1, 1), WF_SEQ(1, 2, 1), WF_SEQ(1, 4, 1),
+      WF_SYN_DS(0), WF_SYN_DS(1), WF_SYN_DS(2), WF_SYN_DS(3), WF_SYN_DS(4),
+      WF_SYN_DS(5), WF_SYN_DS(6), WF_SYN_DS(7), WF_SYN_DS(8),
+  };
+  *n = sizeof(v) / sizeof(v[0]);
+  return v;
+}
+
+const Variant* find(int fn, int dsize, int k, int warps, int skew) {
+  size_t n;
+  const Variant* t = table(&n);
+  for (size_t i = 0; i < n; ++i)
+    if (t[i].fn == fn && t[i].dsize == dsize && t[i].k == k && t[i].warps == warps && t[i].skew == skew) return &t[i];
+  return nullptr;
+}
+
+}  // namespace
+
+bool variant_exists(int fn, int dsize, int k, int warps, int skew) {
+  return find(fn, fn == WF_FN_SYNTHETIC ? dsize : 0, k, warps, skew) != nullptr;
+}
+
+int smem_bytes(const SweepLaunch& L) {
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : 0, L.k, L.warps, L.skew);
+  return v ? (int)v->smem : -1;
+}
+
+int occupancy(const SweepLaunch& L, int smem) {
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : 0, L.k, L.warps, L.skew);
+  if (!v) return 0;
+  if (cudaFuncSetAttribute(v->kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem) != cudaSuccess) {
+    cudaGetLastError();
+    return 0;
+  }
+  int blocks = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, v->kernel, (v->warps + 1) * 32, smem) != cudaSuccess) {
+    cudaGetLastError();
+    return 0;
+  }
+  return blocks;
+}
+
+cudaError_t launch(const SweepLaunch& L, cudaStream_t s) {
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : 0, L.k, L.warps, L.skew);
+  if (!v) return cudaErrorInvalidDeviceFunction;
+  return v->launch(L, s, v->smem);
+}
+
+int variant_count() {
+  size_t n;
+  table(&n);
+  return (int)n;
+}
+
+}  // namespace wfk

@@ -1,0 +1,123 @@
+"""C-ABI boundary tests that need no GPU: the library loads, exports every symbol that
+include/wf.h declares, and validates parameters (WF_EINVAL with a message naming the field).
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+import re
+
+import pytest
+
+from paper_conf_ppopp_mohantyc14_b200 import _abi
+from paper_conf_ppopp_mohantyc14_b200.wf import make_params, query
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+def _declared_symbols():
+    src = open(os.path.join(ROOT, "include", "wf.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(wf_[a-z_]+)\s*\(", src)))
+
+
+def test_library_exports_every_declared_symbol():
+    lib = _abi.lib()
+    declared = _declared_symbols()
+    assert set(declared) == set(_abi.EXPORTS)
+    for name in declared:
+        assert hasattr(lib, name), name
+    assert lib.wf_abi_version() == 1
+    assert b"sm_100a" in lib.wf_build_info()
+
+
+def test_struct_sizes_match_header_layout():
+    # offsets follow the C declaration order with natural alignment
+    assert ctypes.sizeof(_abi.WfParams) == 16 * 4 + 8 + 6 * 4
+    assert ctypes.sizeof(_abi.WfDist) == 16
+    assert _abi.WfParams.watchdog_cycles.offset == 64
+
+
+def _err(fn, dim, **kw):
+    with pytest.raises(_abi.WfError) as ei:
+        query(fn, dim, **kw)
+    return ei.value
+
+
+@pytest.mark.parametrize("kw,field", [
+    (dict(fn="seqcmp", dim=0), "dim"),
+    (dict(fn="seqcmp", dim=70000), "dim"),
+    (dict(fn="seqcmp", dim=100, cols=-3), "cols"),
+    (dict(fn="seqcmp", dim=100, tsize=5), "tsize"),
+    (dict(fn="seqcmp", dim=100, dsize=1), "dsize"),
+    (dict(fn="seqcmp", dim=100, match=100, mismatch=-1, gap=-1), "match"),
+    (dict(fn="seqcmp", dim=100, gap=-65, match=1, mismatch=-1), "gap"),
+    (dict(fn="synthetic", dim=100, dsize=9), "dsize"),
+    (dict(fn="synthetic", dim=100, dsize=1, tsize=-1), "tsize"),
+    (dict(fn="seqcmp", dim=100, lane_cols=3), "lane_cols"),
+    (dict(fn="seqcmp", dim=100, warps=9), "warps"),
+    (dict(fn="seqcmp", dim=100, skew=5), "skew"),
+    (dict(fn="seqcmp", dim=100, ngpus=9), "ngpus"),
+    (dict(fn=7, dim=100), "fn"),
+])
+def test_query_rejects_bad_params_naming_the_field(kw, field):
+    fn = kw.pop("fn")
+    dim = kw.pop("dim")
+    e = _err(fn, dim, **kw)
+    assert e.status == _abi.WF_EINVAL
+    assert field in str(e)
+
+
+def test_reserved_fields_must_be_zero():
+    p = make_params("seqcmp", 64)
+    p.reserved[2] = 1
+    lay = _abi.WfLayout()
+    st = _abi.lib().wf_query(ctypes.byref(p), 0, ctypes.byref(lay))
+    assert st == _abi.WF_EINVAL and b"reserved" in _abi.lib().wf_last_error(None)
+
+
+def test_local_alignment_is_reported_unsupported():
+    e = _err("seqcmp", 64, local=1)
+    assert e.status == _abi.WF_EUNSUPPORTED
+
+
+def test_layout_single_slab():
+    lay = query("seqcmp", 1000, lane_cols=4, warps=2, skew=2)
+    assert (lay.nplanes, lay.col_begin, lay.col_end) == (1, 0, 1000)
+    assert lay.band_cols == 256 and lay.nbands == 4
+    assert lay.min_pitch == 1000 and lay.bytes_out == 1000 * 1000 * 4
+    lay = query("synthetic", 33, tsize=3, dsize=5)
+    assert lay.nplanes == 7 and lay.nbound == 5
+    assert lay.plane_is_float == [False, False, True, True, True, True, True]
+    assert lay.min_pitch == 36
+
+
+@pytest.mark.parametrize("dim,G", [(32768, 8), (1000, 3), (4096, 2), (777, 2)])
+def test_layout_slabs_partition_columns(dim, G):
+    lays = [query("seqcmp", dim, ngpus=G, rank=g) for g in range(G)]
+    assert lays[0].col_begin == 0 and lays[-1].col_end == dim
+    for a, b in zip(lays, lays[1:]):
+        assert a.col_end == b.col_begin
+        # every slab but the last is a whole number of bands
+        assert a.width % a.band_cols == 0
+    assert sum(l.width for l in lays) == dim
+
+
+def test_slab_count_too_large_is_rejected():
+    e = _err("seqcmp", 300, ngpus=4, rank=0, lane_cols=4, warps=2)
+    assert e.status == _abi.WF_EINVAL and "empty" in str(e)
+
+
+def test_null_context_calls_are_rejected():
+    L = _abi.lib()
+    assert L.wf_destroy(None) == _abi.WF_OK
+    assert L.wf_sync(None) == _abi.WF_EINVAL
+    assert L.wf_run(None, None, None) == _abi.WF_EINVAL
+    assert L.wf_last_error(None)  # never NULL
+
+
+def test_create_without_dist_rejects_multi_slab():
+    p = make_params("seqcmp", 128, ngpus=2)
+    ctx = ctypes.c_void_p()
+    st = _abi.lib().wf_create(ctypes.byref(p), None, ctypes.byref(ctx))
+    assert st == _abi.WF_EINVAL and not ctx.value

@@ -1,0 +1,204 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle, element by element.
+
+Bars (BASELINE.json north_star): integer planes bit-exact; fp32 planes
+within |g - o| <= 1e-5 |o| per cell (and, by construction of the fixed op order, expected
+bit-exact -- asserted separately).  Sizes span several bands and ragged tails; the full
+BASELINE configs are covered at the end (C4 full grid; C2 full grid; C5 row prefix plus
+any-size closed forms).
+"""
+from __future__ import annotations
+
+import numpy as np
+import pytest
+
+torch = pytest.importorskip("torch")
+if not torch.cuda.is_available():
+    pytest.skip("needs a CUDA device", allow_module_level=True)
+
+import oracle  # noqa: E402
+import workloads  # noqa: E402
+from paper_conf_ppopp_mohantyc14_b200 import _abi  # noqa: E402
+from paper_conf_ppopp_mohantyc14_b200.wf import Wavefront  # noqa: E402
+
+from _gpu_helpers import dev_inputs, run_gpu  # noqa: E402
+
+pytestmark = pytest.mark.gpu
+
+FTOL = 1e-5
+
+
+def _seq(dim, cols=0, kind="random", scoring=(1, -1, -1), seed=(1, 2), **kw):
+    n = cols or dim
+    x, y = workloads.seqcmp_inputs(dim, n, kind=kind, seed_x=seed[0], seed_y=seed[1])
+    M, X, G = scoring
+    H = oracle.seqcmp(x, y, M, X, G)
+    (g,) = run_gpu("seqcmp", dim, (x, y), cols=cols, match=M, mismatch=X, gap=G, **kw)
+    return H, g
+
+
+# ------------------------------------------------------------------ sequence comparison
+@pytest.mark.parametrize("dim", [1, 2, 3, 7, 31, 32, 33, 63, 64, 65, 100, 127, 129, 255, 256, 257, 500, 512, 1100])
+def test_seqcmp_dims_default_tiling(dim):
+    H, g = _seq(dim)
+    assert np.array_equal(H, g)
+
+
+SEQ_VARIANTS = [(1, 1, 1), (1, 4, 1), (2, 1, 1), (2, 2, 2), (2, 4, 3), (4, 1, 1), (4, 2, 2), (4, 4, 2), (4, 1, 3),
+                (4, 4, 3), (8, 1, 1), (8, 2, 2)]
+
+
+@pytest.mark.parametrize("k,w,d", SEQ_VARIANTS)
+@pytest.mark.parametrize("dim", [97, 777, 1100])
+def test_seqcmp_variants(k, w, d, dim):
+    H, g = _seq(dim, lane_cols=k, warps=w, skew=d, seed=(dim, dim + 1))
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.parametrize("kind", ["identical", "disjoint", "mutated"])
+@pytest.mark.parametrize("scoring", [(1, -1, -1), (1, -1, -2), (2, -3, -1), (5, -4, -10), (64, -64, -64), (0, 0, 1)])
+def test_seqcmp_input_kinds_and_scorings(kind, scoring):
+    H, g = _seq(613, kind=kind, scoring=scoring)
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.parametrize("dim,cols", [(300, 517), (517, 300), (1, 1000), (1000, 1), (2, 3), (33, 4097)])
+def test_seqcmp_rectangular(dim, cols):
+    H, g = _seq(dim, cols=cols)
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.parametrize("max_ctas", [1, 2, 3])
+def test_seqcmp_bands_outnumber_ctas(max_ctas):
+    # persistent loop: CTA i takes bands i, i+grid, ...
+    H, g = _seq(1500, lane_cols=2, warps=1, skew=1, max_ctas=max_ctas)
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.parametrize("G", [2, 3, 4])
+def test_seqcmp_local_slabs_on_one_gpu(G):
+    # G column slabs ("virtual GPUs") on one device, linked through the LL edge rings
+    H, g = _seq(1337, ngpus=G, lane_cols=2, warps=2, skew=2)
+    assert np.array_equal(H, g)
+
+
+def test_seqcmp_rerun_same_context_new_inputs():
+    dim = 700
+    dev = torch.device("cuda")
+    with Wavefront("seqcmp", dim) as w:
+        for seed in range(3):
+            x, y = workloads.seqcmp_inputs(dim, seed_x=10 + seed, seed_y=20 + seed)
+            row_in, col_in, _, _ = dev_inputs("seqcmp", (x, y), dev)
+            out = w.run(row_in, col_in)
+            w.sync()
+            assert np.array_equal(out[0].cpu().numpy(), oracle.seqcmp(x, y))
+        assert w.last_run_ms() > 0
+
+
+def test_seqcmp_determinism_across_tunables():
+    dim = 901
+    x, y = workloads.seqcmp_inputs(dim, seed_x=5, seed_y=6)
+    ref = None
+    for k, w, d in [(1, 1, 1), (2, 4, 3), (4, 2, 2), (8, 1, 2)]:
+        for G in (1, 2):
+            (g,) = run_gpu("seqcmp", dim, (x, y), lane_cols=k, warps=w, skew=d, ngpus=G)
+            if ref is None:
+                ref = g
+            assert np.array_equal(ref, g)
+
+
+def test_watchdog_turns_a_missing_producer_into_a_timeout():
+    # slab 1 of 2 run alone: its west ring is never written -> WF_ETIMEOUT, not a hang
+    dim = 256
+    x, y = workloads.seqcmp_inputs(dim)
+    dev = torch.device("cuda")
+    w = Wavefront("seqcmp", dim, rank=1, device=torch.cuda.current_device(), ngpus=2, lane_cols=1, warps=1,
+                  skew=1, watchdog_cycles=20_000_000)
+    try:
+        row_in, col_in, _, _ = dev_inputs("seqcmp", (x, y), dev)
+        w.run(row_in, col_in)
+        with pytest.raises(_abi.WfError) as ei:
+            w.sync()
+        assert ei.value.status == _abi.WF_ETIMEOUT
+    finally:
+        w.close()
+
+
+def test_seqcmp_c1_config():
+    c = workloads.CONFIGS["C1"]
+    H, g = _seq(c.dim)
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.slow
+def test_seqcmp_c4_full_grid():
+    """C4 (dim=32768) in the launch configuration bench.py times: whole grid bit-exact."""
+    c = workloads.CONFIGS["C4"]
+    H, g = _seq(c.dim)
+    assert np.array_equal(H, g)
+
+
+# ------------------------------------------------------------------ synthetic
+def _syn(dim, tsize, dsize, cols=0, seeds=(3, 4, 5), m_compute=None, **kw):
+    n = cols or dim
+    u, v, top, left = workloads.synthetic_inputs(dim, n, dsize, *seeds)
+    i0, i1, f = oracle.synthetic(u, v, top, left, tsize, m_compute=m_compute)
+    g = run_gpu("synthetic", dim, (u, v, top, left), cols=cols, tsize=tsize, dsize=dsize, **kw)
+    return (i0, i1, f), g
+
+
+def _check_syn(o, g, rows=None):
+    i0, i1, f = o
+    r = slice(0, rows)
+    assert np.array_equal(i0[r], g[0][r])
+    assert np.array_equal(i1[r], g[1][r])
+    for d in range(f.shape[0]):
+        ref, got = f[d][r], g[2 + d][r]
+        assert np.all(np.abs(got - ref) <= FTOL * np.abs(ref)), f"plane f{d} exceeds 1e-5 relative"
+        assert np.array_equal(ref.view(np.uint32), got.view(np.uint32)), f"plane f{d} not bit-exact"
+
+
+@pytest.mark.parametrize("dim", [1, 2, 31, 33, 100, 257])
+@pytest.mark.parametrize("tsize", [0, 1, 10, 100])
+@pytest.mark.parametrize("dsize", [0, 1, 2, 5, 8])
+def test_synthetic_grid(dim, tsize, dsize):
+    o, g = _syn(dim, tsize, dsize)
+    _check_syn(o, g)
+
+
+@pytest.mark.parametrize("k,w,d", [(1, 1, 1), (1, 4, 1), (2, 1, 1), (2, 2, 1), (1, 2, 2), (2, 2, 2)])
+def test_synthetic_variants(k, w, d):
+    o, g = _syn(419, 7, 3, lane_cols=k, warps=w, skew=d)
+    _check_syn(o, g)
+
+
+@pytest.mark.parametrize("G", [2, 3])
+def test_synthetic_local_slabs(G):
+    o, g = _syn(333, 5, 2, ngpus=G)
+    _check_syn(o, g)
+
+
+def test_synthetic_rectangular():
+    o, g = _syn(129, 3, 2, cols=300)
+    _check_syn(o, g)
+
+
+def test_synthetic_c2_full_grid():
+    c = workloads.CONFIGS["C2"]
+    o, g = _syn(c.dim, c.tsize, c.dsize)
+    _check_syn(o, g)
+
+
+@pytest.mark.slow
+@pytest.mark.parametrize("name,prefix", [("C5a", 64), ("C5b", 32), ("C5c", 8), ("C5d", 4)])
+def test_synthetic_c5_prefix_and_closed_forms(name, prefix):
+    """C5 at full size: exact parity on a row prefix (a true prefix of the grid), plus the
+    closed forms i0 = (i-1)+(j-1), i1 = i*j and the value range on EVERY cell."""
+    c = workloads.CONFIGS[name]
+    o, g = _syn(c.dim, c.tsize, c.dsize, m_compute=prefix)
+    _check_syn(o, g, rows=prefix)
+    i = np.arange(1, c.dim + 1, dtype=np.int64)[:, None]
+    j = np.arange(1, c.dim + 1, dtype=np.int64)[None, :]
+    assert np.array_equal(g[0], (i - 1) + (j - 1))
+    assert np.array_equal(g[1], (i * j).astype(np.int64).astype(np.int32))
+    for d in range(c.dsize):
+        assert g[2 + d].min() >= 0.25 and g[2 + d].max() < 1.0
