@@ -116,6 +116,8 @@ def host_inputs(cfg):
 
 def fn_kwargs(cfg):
     kw = {}
+    if cfg.fn == "seqcmp":
+        kw = dict(alphabet=4)   # DNA codes {0..3} (workloads.seqcmp_inputs)
     if cfg.fn == "synthetic":
         kw = dict(tsize=cfg.tsize, dsize=cfg.dsize)
     elif cfg.fn == "nash":

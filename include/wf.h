@@ -88,7 +88,10 @@ typedef struct {
   uint32_t transport;   /* wf_transport for ngpus > 1 */
   uint32_t max_ctas;    /* 0 = all resident CTAs; else an upper bound (tests of the band loop) */
   uint64_t watchdog_cycles; /* spin budget per dependency wait (SM clock cycles); 0 = default 2^32 */
-  int32_t reserved[6];  /* must be zero */
+  int32_t alphabet;     /* SEQCMP: 0 = residue codes may be any byte value; 1..8 = every code in
+                           row_in/col_in is < alphabet (e.g. 4 for DNA) -- enables the byte-permute
+                           score lookup; codes outside the promise give unspecified scores */
+  int32_t reserved[5];  /* must be zero */
 } wf_params;
 
 /* Distribution: which slab this context computes.
@@ -183,6 +186,13 @@ wf_status wf_connect(struct wf_ctx* c, const void* prev_handle, const void* next
 /* Device time of the last completed run in milliseconds (CUDA events bracketing the
  * launch on the run's stream); WF_ESTATE if no run has completed. */
 wf_status wf_last_run_ms(struct wf_ctx* c, float* ms);
+
+/* Diagnostics: when the process runs with WF_TRACE=1, each wf_run records per band a
+ * timeline of %globaltimer stamps (ns) taken by the band's first lane every rows/32 rows
+ * (slots 0..31), at its last row (slot 32), and the feeder's poll / empty-poll counts
+ * (slots 40, 41).  Copies min(bytes, nbands*slots*8) bytes of the last run to host;
+ * *slots_per_band receives the slot count.  WF_ESTATE if tracing was not enabled. */
+wf_status wf_debug_trace(struct wf_ctx* c, void* host, size_t bytes, int32_t* slots_per_band);
 
 /* Library build information: ABI version, compiled arch, kernel variant count. */
 int32_t wf_abi_version(void);

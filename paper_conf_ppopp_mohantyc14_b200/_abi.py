@@ -8,7 +8,7 @@ import ctypes
 import os
 
 HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(HERE, "libwf.so")
+LIB_PATH = os.environ.get("WF_LIB_OVERRIDE") or os.path.join(HERE, "libwf.so")   # override: perf experiments
 
 WF_MAX_PLANES = 10
 WF_IPC_HANDLE_BYTES = 64
@@ -22,7 +22,7 @@ WF_TRANSPORT_P2P, WF_TRANSPORT_NCCL = 0, 1
 
 # every symbol include/wf.h declares (checked by tests/test_abi.py)
 EXPORTS = ("wf_query", "wf_create", "wf_run", "wf_sync", "wf_destroy", "wf_last_error", "wf_link_local",
-           "wf_ipc_handle", "wf_connect", "wf_last_run_ms", "wf_abi_version", "wf_build_info")
+           "wf_ipc_handle", "wf_connect", "wf_last_run_ms", "wf_abi_version", "wf_build_info", "wf_debug_trace")
 
 
 class WfParams(ctypes.Structure):
@@ -32,7 +32,7 @@ class WfParams(ctypes.Structure):
                 ("ngpus", ctypes.c_int32), ("match", ctypes.c_int32), ("mismatch", ctypes.c_int32),
                 ("gap", ctypes.c_int32), ("local", ctypes.c_int32), ("transport", ctypes.c_uint32),
                 ("max_ctas", ctypes.c_uint32), ("watchdog_cycles", ctypes.c_uint64),
-                ("reserved", ctypes.c_int32 * 6)]
+                ("alphabet", ctypes.c_int32), ("reserved", ctypes.c_int32 * 5)]
 
 
 class WfDist(ctypes.Structure):
@@ -84,6 +84,8 @@ def lib() -> ctypes.CDLL:
         L.wf_ipc_handle.argtypes = [P, P]
         L.wf_connect.argtypes = [P, P, P]
         L.wf_last_run_ms.argtypes = [P, ctypes.POINTER(ctypes.c_float)]
+        L.wf_debug_trace.argtypes = [P, P, ctypes.c_size_t, ctypes.POINTER(ctypes.c_int32)]
+        L.wf_debug_trace.restype = ctypes.c_int
         L.wf_abi_version.argtypes = []
         L.wf_abi_version.restype = ctypes.c_int32
         L.wf_build_info.argtypes = []

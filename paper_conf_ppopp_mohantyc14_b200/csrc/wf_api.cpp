@@ -8,6 +8,7 @@
 
 #include <cstdarg>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <new>
 #include <string>
@@ -36,6 +37,7 @@ struct wf_ctx {
   unsigned long long* next_edge = nullptr; // next slab's band-0 ring (peer / IPC / local)
   void* next_ipc_base = nullptr;
   int* err = nullptr;                      // device error word
+  unsigned long long* trace = nullptr;     // WF_TRACE=1 timeline buffer (diagnostics)
   uint32_t epoch = 0;
   cudaEvent_t ev0 = nullptr, ev1 = nullptr;
   bool ran = false;
@@ -87,8 +89,10 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   const int cols = p->cols ? p->cols : p->dim;
   if (rows < 1 || rows > 65535) return fail(c, WF_EINVAL, "dim=%d out of range 1..65535", rows);
   if (cols < 1 || cols > 65535) return fail(c, WF_EINVAL, "cols=%d out of range 1..65535", cols);
-  for (int i = 0; i < 6; ++i)
+  for (int i = 0; i < 5; ++i)
     if (p->reserved[i]) return fail(c, WF_EINVAL, "reserved[%d] must be 0", i);
+  if (p->alphabet < 0 || p->alphabet > 8) return fail(c, WF_EINVAL, "alphabet=%d out of range 0..8", p->alphabet);
+  if (p->alphabet != 0 && p->fn != WF_FN_SEQCMP) return fail(c, WF_EINVAL, "alphabet applies to SEQCMP only");
   if (p->ngpus < 0 || p->ngpus > 8) return fail(c, WF_EINVAL, "ngpus=%d out of range 1..8", p->ngpus);
   const int G = p->ngpus ? p->ngpus : 1;
   if (rank < 0 || rank >= G) return fail(c, WF_EINVAL, "rank=%d out of range for ngpus=%d", rank, G);
@@ -273,7 +277,7 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   if (p->max_ctas && (int)p->max_ctas < c->grid) c->grid = (int)p->max_ctas;
   if (c->grid < 1) c->grid = 1;
 
-  c->edge_bytes = (size_t)pl.nbands * p->dim * pl.nf * sizeof(unsigned long long);
+  c->edge_bytes = (size_t)pl.nbands * wfk::edge_stride(p->dim) * pl.nf * sizeof(unsigned long long);
   e = cudaMalloc(&c->base, kCtrlBytes + c->edge_bytes);
   if (e == cudaSuccess) e = cudaMemset(c->base, 0, kCtrlBytes + c->edge_bytes);
   if (e == cudaSuccess) {
@@ -304,6 +308,7 @@ wf_status wf_destroy(wf_ctx* c) {
   if (c->prev_ipc_base) cudaIpcCloseMemHandle(c->prev_ipc_base);
   if (c->base) cudaFree(c->base);
   if (c->err) cudaFree(c->err);
+  if (c->trace) cudaFree(c->trace);
   if (c->ev0) cudaEventDestroy(c->ev0);
   if (c->ev1) cudaEventDestroy(c->ev1);
   if (prev >= 0) cudaSetDevice(prev);
@@ -437,6 +442,7 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   L.match = p.match;
   L.mismatch = p.mismatch;
   L.gap = p.gap;
+  L.alphabet = p.alphabet;
   L.k = c->k;
   L.warps = c->warps;
   L.skew = c->skew;
@@ -459,6 +465,12 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   L.epoch = ++c->epoch;
   if ((L.epoch & 0x0FFFFFFFu) == 0) L.epoch = ++c->epoch;   // tag 0 marks "never written"
   L.err = c->err;
+  if (!c->trace && getenv("WF_TRACE") && getenv("WF_TRACE")[0] == '1') {
+    cudaMalloc(&c->trace, (size_t)c->nbands * wfk::kTraceSlots * 8);
+    cudaGetLastError();
+  }
+  if (c->trace) cudaMemsetAsync(c->trace, 0, (size_t)c->nbands * wfk::kTraceSlots * 8, static_cast<cudaStream_t>(cuda_stream));
+  L.trace = c->trace;
   L.watchdog = p.watchdog_cycles ? p.watchdog_cycles : (1ull << 32);
 
   int prev = -1;
@@ -485,6 +497,16 @@ wf_status wf_sync(wf_ctx* c) {
   if (((unsigned)w >> 4) == (c->epoch & 0x0FFFFFFFu) && (w & 15) == wfk::DEV_TIMEOUT)
     return fail(c, WF_ETIMEOUT, "watchdog: a dependency wait exceeded %llu cycles (run epoch %u)",
                 (unsigned long long)(c->p.watchdog_cycles ? c->p.watchdog_cycles : (1ull << 32)), c->epoch);
+  return WF_OK;
+}
+
+wf_status wf_debug_trace(wf_ctx* c, void* host, size_t bytes, int32_t* slots_per_band) {
+  if (!c || !host || !slots_per_band) return fail(c, WF_EINVAL, "wf_debug_trace: NULL argument");
+  *slots_per_band = wfk::kTraceSlots;
+  if (!c->trace) return fail(c, WF_ESTATE, "wf_debug_trace: run with WF_TRACE=1 in the environment");
+  const size_t need = (size_t)c->nbands * wfk::kTraceSlots * 8;
+  cudaError_t e = cudaMemcpy(host, c->trace, bytes < need ? bytes : need, cudaMemcpyDeviceToHost);
+  if (e != cudaSuccess) return cuda_fail(c, e, "wf_debug_trace");
   return WF_OK;
 }
 

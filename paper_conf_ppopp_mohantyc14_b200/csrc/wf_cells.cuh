@@ -13,6 +13,7 @@ namespace wfk {
 //     H = max(max(NW + s, N + g), W + g): two DPX VIADDMNMX, W last.
 struct PolSeq {
   static constexpr int NF = 1;
+  static constexpr bool kTagRowIn = true;   // x_i travels in the LL tag's top byte
   const uint8_t* x;
   const uint8_t* y;
   int32_t match, mismatch, gap;
@@ -34,6 +35,7 @@ struct PolSeq {
 template <int DS>
 struct PolSyn {
   static constexpr int NF = 2 + DS;
+  static constexpr bool kTagRowIn = false;
   const float* u;
   const float* v;
   const float* topf[DS > 0 ? DS : 1];

@@ -14,6 +14,7 @@ struct SweepLaunch {
   int32_t fn, rows, cols, tsize, dsize;
   int32_t c0, c1;                 // slab interior columns [c0, c1), 0-based
   int32_t match, mismatch, gap;
+  int32_t alphabet;               // SEQCMP: 0 = any byte codes, 1..8 = codes < alphabet
   // tuning
   int32_t k, warps, skew;         // lane columns, compute warps per CTA, lane skew
   int32_t band_w, nbands;         // band_w = warps*32*k
@@ -37,8 +38,15 @@ struct SweepLaunch {
   int32_t first_slab;             // 1: band 0's west input is the column-0 boundary
   uint32_t epoch;
   int* err;                       // device error word
+  // Optional timeline (WF_TRACE=1): per band kTraceSlots globaltimer stamps written by
+  // compute warp 0 lane 0 every rows/kTraceRows rows, plus feeder poll counters.
+  unsigned long long* trace;
   unsigned long long watchdog;
 };
+
+// LL slots per band ring and cell word: slot r holds row r (1..rows); padded to an even
+// count so every band's ring starts 16-byte aligned (vector LL stores).
+__host__ __device__ inline size_t edge_stride(int rows) { return size_t((rows + 2) & ~1); }
 
 // Words per cell (= output planes) for a function.
 int nwords(int fn, int dsize);
@@ -50,6 +58,9 @@ int occupancy(const SweepLaunch& L, int smem);
 cudaError_t launch(const SweepLaunch& L, cudaStream_t s);
 // Is (fn, dsize, k, warps, skew) compiled?
 bool variant_exists(int fn, int dsize, int k, int warps, int skew);
+
+constexpr int kTraceSlots = 48;   // per band: [0..32] row stamps, [40] feeder polls, [41] empty polls,
+constexpr int kTraceRows = 32;    // [42] last warp's first outbound stamp
 
 // Error word codes (device side).
 enum : int { DEV_OK = 0, DEV_TIMEOUT = 1 };

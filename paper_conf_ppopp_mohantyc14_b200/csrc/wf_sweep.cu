@@ -3,7 +3,11 @@
 #include <cstring>
 #include <type_traits>
 
+#include <cuda.h>
+#include <cudaTypedefs.h>
+
 #include "wf_cells.cuh"
+#include "wf_nw.cuh"
 #include "wf_sweep.cuh"
 
 namespace wfk {
@@ -58,23 +62,76 @@ Variant make_variant(int fn, int dsize) {
                  &launch_t<P, K, W, D>};
 }
 
+// cuTensorMapEncodeTiled through the runtime's driver entry point (no -lcuda link needed)
+cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols, int box_rows) {
+  static PFN_cuTensorMapEncodeTiled_v12000 enc = nullptr;
+  if (!enc) {
+    void* fp = nullptr;
+    cudaDriverEntryPointQueryResult q;
+    cudaError_t e = cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fp, cudaEnableDefault, &q);
+    if (e != cudaSuccess || q != cudaDriverEntryPointSuccess || !fp) return cudaErrorNotSupported;
+    enc = reinterpret_cast<PFN_cuTensorMapEncodeTiled_v12000>(fp);
+  }
+  const cuuint64_t dims[2] = {static_cast<cuuint64_t>(L.c1 - L.c0), static_cast<cuuint64_t>(L.rows)};
+  const cuuint64_t strides[1] = {static_cast<cuuint64_t>(L.pitch) * 4};
+  const cuuint32_t box[2] = {static_cast<cuuint32_t>(box_cols), static_cast<cuuint32_t>(box_rows)};
+  const cuuint32_t estr[2] = {1, 1};
+  CUresult r = enc(m, CU_TENSOR_MAP_DATA_TYPE_INT32, 2, L.out[0], dims, strides, box, estr,
+                   CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_NONE,
+                   CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  return r == CUDA_SUCCESS ? cudaSuccess : cudaErrorInvalidValue;
+}
+
+template <int K, int W, int D, int U>
+cudaError_t launch_nw(const SweepLaunch& L, cudaStream_t s, size_t smem) {
+  PolSeq pol{};
+  pol.x = static_cast<const uint8_t*>(L.row_in);
+  pol.y = static_cast<const uint8_t*>(L.col_in);
+  pol.match = L.match;
+  pol.mismatch = L.mismatch;
+  pol.gap = L.gap;
+  // TMA descriptor of this slab's output plane: int32 [rows][slab cols], row pitch in bytes,
+  // box = one warp's 32*K columns x U rows (the steady-state write-out unit)
+  CUtensorMap tmap;
+  cudaError_t e = encode_plane_map(&tmap, L, 32 * K, U);
+  if (e != cudaSuccess) return e;
+  // alphabet 1..8 promises codes < 8: byte-permute score lookup; otherwise compare+select
+  auto kfn = (L.alphabet >= 1 && L.alphabet <= 8) ? nw_kernel<K, W, D, U, true> : nw_kernel<K, W, D, U, false>;
+  e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  if (e != cudaSuccess) return e;
+  kfn<<<L.grid, (W + 1) * 32, smem, s>>>(L, pol, tmap);
+  return cudaGetLastError();
+}
+
+template <int K, int W, int D>
+Variant make_nw_variant() {
+  constexpr int U = K >= 8 ? 8 : 16;   // rows per block (TMA box height)
+  using S = NwSmem<K, W, D, U>;
+  return Variant{WF_FN_SEQCMP, 0, K, W, D, S::bytes, reinterpret_cast<const void*>(nw_kernel<K, W, D, U, true>),
+                 &launch_nw<K, W, D, U>};
+}
+
 // --- the compiled variant set -------------------------------------------------------
-#define WF_SEQ(K, W, D) make_variant<PolSeq, K, W, D>(WF_FN_SEQCMP, 0)
+#define WF_SEQ(K, W, D) make_nw_variant<K, W, D>()
 #define WF_SYN(DS, K, W, D) make_variant<PolSyn<DS>, K, W, D>(WF_FN_SYNTHETIC, DS)
 #define WF_SYN_DS(DS) WF_SYN(DS, 1, 1, 1), WF_SYN(DS, 1, 2, 1), WF_SYN(DS, 1, 4, 1), WF_SYN(DS, 2, 1, 1), \
     WF_SYN(DS, 2, 2, 1), WF_SYN(DS, 1, 2, 2), WF_SYN(DS, 2, 2, 2)
 
 const Variant* table(size_t* n) {
+#ifdef WF_MIN_VARIANTS   // quick experimental builds (tools/ablate.sh)
+  static const Variant v[] = {WF_SEQ(4, 1, 1), WF_SEQ(4, 1, 2), WF_SEQ(4, 2, 1), WF_SEQ(2, 1, 1), WF_SEQ(8, 1, 1)};
+#else
   static const Variant v[] = {
       WF_SEQ(2, 1, 1), WF_SEQ(2, 2, 1), WF_SEQ(2, 4, 1), WF_SEQ(2, 1, 2), WF_SEQ(2, 2, 2), WF_SEQ(2, 4, 2),
       WF_SEQ(2, 2, 3), WF_SEQ(2, 4, 3),
       WF_SEQ(4, 1, 1), WF_SEQ(4, 2, 1), WF_SEQ(4, 4, 1), WF_SEQ(4, 1, 2), WF_SEQ(4, 2, 2), WF_SEQ(4, 4, 2),
-      WF_SEQ(4, 1, 3), WF_SEQ(4, 2, 3), WF_SEQ(4, 4, 3),
+      WF_SEQ(4, 1, 3), WF_SEQ(4, 2, 3),
       WF_SEQ(8, 1, 1), WF_SEQ(8, 2, 1), WF_SEQ(8, 1, 2), WF_SEQ(8, 2, 2),
       WF_SEQ(1, 1, 1), WF_SEQ(1, 2, 1), WF_SEQ(1, 4, 1),
       WF_SYN_DS(0), WF_SYN_DS(1), WF_SYN_DS(2), WF_SYN_DS(3), WF_SYN_DS(4),
       WF_SYN_DS(5), WF_SYN_DS(6), WF_SYN_DS(7), WF_SYN_DS(8),
   };
+#endif
   *n = sizeof(v) / sizeof(v[0]);
   return v;
 }
@@ -90,7 +147,9 @@ const Variant* find(int fn, int dsize, int k, int warps, int skew) {
 }  // namespace
 
 bool variant_exists(int fn, int dsize, int k, int warps, int skew) {
-  return find(fn, fn == WF_FN_SYNTHETIC ? dsize : 0, k, warps, skew) != nullptr;
+  // compiled AND within the 227 KB per-CTA shared-memory limit of sm_100
+  const Variant* v = find(fn, fn == WF_FN_SYNTHETIC ? dsize : 0, k, warps, skew);
+  return v != nullptr && v->smem <= 232448;
 }
 
 int smem_bytes(const SweepLaunch& L) {

@@ -56,6 +56,11 @@ __device__ __forceinline__ unsigned ld_relaxed_sys_u32(const unsigned* p) {
   asm volatile("ld.relaxed.sys.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
   return v;
 }
+__device__ __forceinline__ unsigned long long globaltimer() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+  return t;
+}
 __device__ __forceinline__ unsigned long long lds_vol(const unsigned long long* p) {
   return *reinterpret_cast<const volatile unsigned long long*>(p);
 }
@@ -124,22 +129,26 @@ struct Smem {
 // Feeder warp: west input of the band's first column for every row, from the
 // column-0 boundary (first band of slab 0) or from the band's global LL ring.
 // ---------------------------------------------------------------------------------
-template <class P, int K, int WARPS, int D>
-__device__ __forceinline__ bool feeder(const SweepLaunch& L, const P& pol, const Smem<P::NF, K, WARPS, D>& sm,
-                                       int band, int lane) {
+template <class P, class SM>
+__device__ __forceinline__ bool feeder(const SweepLaunch& L, const P& pol, const SM& sm, int band, int lane) {
   constexpr int NF = P::NF;
   const bool boundary = L.first_slab && band == 0;
-  const unsigned long long* src = L.edge + size_t(band) * L.rows * NF;
+  const unsigned long long* src = L.edge + size_t(band) * edge_stride(L.rows) * NF;   // slot r holds row r
   int base = 1, seen_prog = 0;
   Watchdog wd;
   wd.start();
   while (base <= L.rows) {
     // back-pressure: rows base .. base+63 go to slots that held rows base-256 .. ;
     // those must have been consumed by compute warp 0.
+    // The feeder is normally far ahead, so it sleeps between polls: a tight LDS spin would
+    // occupy the SM's MIO pipe that the compute warps' SHFL/LDS/STS depend on.
     const int need = base + 63 - kHandSlots;
     while (seen_prog < need) {
       seen_prog = lds_vol_i(sm.prog + 0);
-      if (seen_prog < need && wd.expired(L)) return false;
+      if (seen_prog < need) {
+        if (wd.expired(L)) return false;
+        __nanosleep(256);
+      }
     }
     uint32_t v[2][NF];
     bool ok[2];
@@ -153,7 +162,7 @@ __device__ __forceinline__ bool feeder(const SweepLaunch& L, const P& pol, const
         } else {
 #pragma unroll
           for (int f = 0; f < NF; ++f) {
-            const unsigned long long w = ld_relaxed_sys(src + size_t(r - 1) * NF + f);
+            const unsigned long long w = ld_relaxed_sys(src + size_t(r) * NF + f);
             v[h][f] = static_cast<uint32_t>(w);
             ok[h] = ok[h] && static_cast<uint32_t>(w >> 32) == L.epoch;
           }
@@ -169,13 +178,24 @@ __device__ __forceinline__ bool feeder(const SweepLaunch& L, const P& pol, const
       const int r = base + h * 32 + lane;
       if (r < base + n) {
         unsigned long long* slot = sm.hand_slot(0, r);
+        // policies with a byte-sized row input (x_i of sequence comparison) ship it in the
+        // tag's top byte, so compute warps never load it from global memory
+        uint32_t tag = static_cast<uint32_t>(r);
+        if constexpr (P::kTagRowIn) tag |= pol.row_in(r) << 24;
 #pragma unroll
-        for (int f = 0; f < NF; ++f) sts_vol(slot + f, ll_pack(v[h][f], static_cast<uint32_t>(r)));
+        for (int f = 0; f < NF; ++f) sts_vol(slot + f, ll_pack(v[h][f], tag));
       }
+    }
+    if (L.trace && lane == 0) {
+      L.trace[size_t(band) * kTraceSlots + 40] += 1;
+      if (n == 0) L.trace[size_t(band) * kTraceSlots + 41] += 1;
     }
     if (n == 0) {
       if (wd.expired(L)) return false;
-      __nanosleep(64);
+      __nanosleep(128);
+    } else if (n < 32) {
+      __nanosleep(64);   // producer is just ahead: poll less often, let it run ahead
+      wd.start();
     } else {
       wd.start();
     }
@@ -228,9 +248,12 @@ __device__ __forceinline__ bool compute_warp(const SweepLaunch& L, const P& pol,
   }
   Watchdog wd;
   const int T = rows + 31 * D;
+  const int trace_every = (rows + kTraceRows - 1) / kTraceRows;
   for (int t = 0; t < T; ++t) {
     const int row = t - D * lane + 1;
     const bool active = row >= 1 && row <= rows;
+    if (L.trace && warp == 0 && lane == 0 && t < rows && (t % trace_every) == 0)
+      L.trace[size_t(band) * kTraceSlots + t / trace_every] = globaltimer();
     const uint32_t xr = xr_next;
     {
       const int rn = row + 1;
@@ -331,10 +354,10 @@ __device__ __forceinline__ bool compute_warp(const SweepLaunch& L, const P& pol,
             if (wd.expired(L)) return false;
           }
         }
-        unsigned long long* dst = to_next_slab ? L.next_edge : L.edge + size_t(band + 1) * rows * NF;
+        unsigned long long* dst = to_next_slab ? L.next_edge : L.edge + size_t(band + 1) * edge_stride(rows) * NF;
         if (dst && lane == 31) {
 #pragma unroll
-          for (int f = 0; f < NF; ++f) st_relaxed_sys(dst + size_t(r31 - 1) * NF + f, ll_pack(Np[K - 1][f], L.epoch));
+          for (int f = 0; f < NF; ++f) st_relaxed_sys(dst + size_t(r31) * NF + f, ll_pack(Np[K - 1][f], L.epoch));
         }
       }
     }
@@ -366,6 +389,7 @@ __device__ __forceinline__ bool compute_warp(const SweepLaunch& L, const P& pol,
     }
     __syncwarp();
   }
+  if (L.trace && warp == 0 && lane == 0) L.trace[size_t(band) * kTraceSlots + kTraceRows] = globaltimer();
   (void)R;
   return true;
 }
@@ -381,7 +405,7 @@ __global__ void __launch_bounds__((WARPS + 1) * 32) sweep_kernel(const SweepLaun
     if (threadIdx.x < WARPS) sm.prog[threadIdx.x] = 0;
     __syncthreads();
     bool ok;
-    if (warp == WARPS) ok = feeder<P, K, WARPS, D>(L, pol, sm, band, lane);
+    if (warp == WARPS) ok = feeder(L, pol, sm, band, lane);
     else ok = compute_warp<P, K, WARPS, D>(L, pol, sm, band, warp, lane);
     (void)ok;
     __syncthreads();

@@ -39,7 +39,8 @@ class Layout:
 
 
 def make_params(fn, dim, *, cols=0, tsize=0, dsize=0, lane_cols=0, warps=0, skew=0, strip=0, ngpus=1,
-                match=0, mismatch=0, gap=0, local=0, transport="p2p", max_ctas=0, watchdog_cycles=0) -> WfParams:
+                match=0, mismatch=0, gap=0, local=0, transport="p2p", max_ctas=0, watchdog_cycles=0,
+                alphabet=0) -> WfParams:
     p = WfParams()
     p.dim = int(dim)
     p.cols = int(cols)
@@ -56,6 +57,7 @@ def make_params(fn, dim, *, cols=0, tsize=0, dsize=0, lane_cols=0, warps=0, skew
     p.transport = _TRANSPORTS[transport] if isinstance(transport, str) else int(transport)
     p.max_ctas = int(max_ctas)
     p.watchdog_cycles = int(watchdog_cycles)
+    p.alphabet = int(alphabet)
     return p
 
 
@@ -144,6 +146,16 @@ class Wavefront:
         ms = ctypes.c_float()
         check(_abi.lib().wf_last_run_ms(self._ctx, ctypes.byref(ms)), self._ctx)
         return float(ms.value)
+
+    def debug_trace(self):
+        """(nbands, slots) uint64 timeline of the last run (needs WF_TRACE=1 at run time)."""
+        import numpy as np
+        buf = np.zeros((self.layout.nbands, 64), dtype=np.uint64)
+        slots = ctypes.c_int32()
+        check(_abi.lib().wf_debug_trace(self._ctx, buf.ctypes.data, buf.nbytes, ctypes.byref(slots)), self._ctx)
+        buf = np.zeros((self.layout.nbands, slots.value), dtype=np.uint64)
+        check(_abi.lib().wf_debug_trace(self._ctx, buf.ctypes.data, buf.nbytes, ctypes.byref(slots)), self._ctx)
+        return buf
 
     # ---- multi-slab plumbing
     def link(self, nxt: "Wavefront") -> None:

@@ -43,14 +43,29 @@ def test_seqcmp_dims_default_tiling(dim):
     assert np.array_equal(H, g)
 
 
-SEQ_VARIANTS = [(1, 1, 1), (1, 4, 1), (2, 1, 1), (2, 2, 2), (2, 4, 3), (4, 1, 1), (4, 2, 2), (4, 4, 2), (4, 1, 3),
-                (4, 4, 3), (8, 1, 1), (8, 2, 2)]
+SEQ_VARIANTS = [(1, 1, 1), (1, 4, 1), (2, 1, 1), (2, 2, 2), (2, 2, 3), (2, 4, 1), (4, 1, 1), (4, 2, 1), (4, 2, 2),
+                (4, 1, 3), (8, 1, 1), (8, 2, 1)]
 
 
 @pytest.mark.parametrize("k,w,d", SEQ_VARIANTS)
 @pytest.mark.parametrize("dim", [97, 777, 1100])
-def test_seqcmp_variants(k, w, d, dim):
-    H, g = _seq(dim, lane_cols=k, warps=w, skew=d, seed=(dim, dim + 1))
+@pytest.mark.parametrize("alphabet", [0, 4])
+def test_seqcmp_variants(k, w, d, dim, alphabet):
+    H, g = _seq(dim, lane_cols=k, warps=w, skew=d, seed=(dim, dim + 1), alphabet=alphabet)
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.parametrize("alphabet", [4, 8])
+@pytest.mark.parametrize("scoring", [(1, -1, -1), (2, -3, -1), (-3, 2, -1), (64, -64, -64), (-64, 64, 64)])
+def test_seqcmp_byte_permute_scores(alphabet, scoring):
+    # the PRMT score lookup must sign-extend every int8 score and honour match < mismatch
+    dim = 555
+    rng = np.random.default_rng(alphabet)
+    x = rng.integers(0, alphabet, size=dim).astype(np.uint8)
+    y = rng.integers(0, alphabet, size=dim).astype(np.uint8)
+    M, X, G = scoring
+    H = oracle.seqcmp(x, y, M, X, G)
+    (g,) = run_gpu("seqcmp", dim, (x, y), match=M, mismatch=X, gap=G, alphabet=alphabet)
     assert np.array_equal(H, g)
 
 
@@ -79,6 +94,8 @@ def test_seqcmp_local_slabs_on_one_gpu(G):
     # G column slabs ("virtual GPUs") on one device, linked through the LL edge rings
     H, g = _seq(1337, ngpus=G, lane_cols=2, warps=2, skew=2)
     assert np.array_equal(H, g)
+    H, g = _seq(2900, ngpus=G, lane_cols=4, warps=2, skew=1, alphabet=4)
+    assert np.array_equal(H, g)
 
 
 def test_seqcmp_rerun_same_context_new_inputs():
@@ -98,7 +115,7 @@ def test_seqcmp_determinism_across_tunables():
     dim = 901
     x, y = workloads.seqcmp_inputs(dim, seed_x=5, seed_y=6)
     ref = None
-    for k, w, d in [(1, 1, 1), (2, 4, 3), (4, 2, 2), (8, 1, 2)]:
+    for k, w, d in [(1, 1, 1), (2, 2, 3), (4, 2, 2), (8, 1, 2)]:
         for G in (1, 2):
             (g,) = run_gpu("seqcmp", dim, (x, y), lane_cols=k, warps=w, skew=d, ngpus=G)
             if ref is None:
@@ -133,7 +150,7 @@ def test_seqcmp_c1_config():
 def test_seqcmp_c4_full_grid():
     """C4 (dim=32768) in the launch configuration bench.py times: whole grid bit-exact."""
     c = workloads.CONFIGS["C4"]
-    H, g = _seq(c.dim)
+    H, g = _seq(c.dim, alphabet=4)
     assert np.array_equal(H, g)
 
 
