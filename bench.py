@@ -351,7 +351,7 @@ def run_ours(args, cfg):
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
                          "traffic": traffic, "peak_source": peak_src,
                          "algorithmic_bytes_per_launch": bytes_per_launch, "avg_launch_ms": avg_launch_ms,
-                         "kernel": "wfk::sweep_kernel"},
+                         "kernel": "wfk::nw_kernel" if cfg.fn == "seqcmp" else "wfk::sweep_kernel"},
             "e2e": {"value": total_cells / (e2e_ms * 1e-3) / 1e9, "unit": UNIT, "ms_per_step": e2e_ms,
                     "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                     "note": "H2D of the step's inputs from pinned memory, sweep, D2H of the result row"},

@@ -75,7 +75,7 @@ void defaults(const wf_params& p, int* k, int* w, int* d) {
   if (p.fn == WF_FN_SEQCMP) {
     *k = p.lane_cols ? p.lane_cols : 4;
     *w = p.warps ? p.warps : 2;
-    *d = p.skew ? p.skew : 2;
+    *d = p.skew ? p.skew : 1;
   } else {
     *k = p.lane_cols ? p.lane_cols : 1;
     *w = p.warps ? p.warps : 2;
