@@ -59,7 +59,7 @@ cudaError_t launch(const SweepLaunch& L, cudaStream_t s);
 // Is (fn, dsize, k, warps, skew) compiled?
 bool variant_exists(int fn, int dsize, int k, int warps, int skew);
 
-constexpr int kTraceSlots = 48;   // per band: [0..32] row stamps, [40] feeder polls, [41] empty polls,
+constexpr int kTraceSlots = 64;   // per band: [0..32] row stamps, [40] feeder polls, [41] empty polls,
 constexpr int kTraceRows = 32;    // [42] last warp's first outbound stamp
 
 // Error word codes (device side).

@@ -25,6 +25,7 @@ namespace {
 
 struct Variant {
   int fn, dsize, k, warps, skew;
+  int threads;         // CTA size (compute warps + helper warps)
   size_t smem;
   const void* kernel;  // __global__ function pointer (for occupancy queries)
   cudaError_t (*launch)(const SweepLaunch&, cudaStream_t, size_t);
@@ -58,7 +59,7 @@ cudaError_t launch_t(const SweepLaunch& L, cudaStream_t s, size_t smem) {
 template <class P, int K, int W, int D>
 Variant make_variant(int fn, int dsize) {
   using S = Smem<P::NF, K, W, D>;
-  return Variant{fn, dsize, K, W, D, S::bytes, reinterpret_cast<const void*>(sweep_kernel<P, K, W, D>),
+  return Variant{fn, dsize, K, W, D, (W + 1) * 32, S::bytes, reinterpret_cast<const void*>(sweep_kernel<P, K, W, D>),
                  &launch_t<P, K, W, D>};
 }
 
@@ -99,15 +100,19 @@ cudaError_t launch_nw(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   auto kfn = (L.alphabet >= 1 && L.alphabet <= 8) ? nw_kernel<K, W, D, U, true> : nw_kernel<K, W, D, U, false>;
   e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
-  kfn<<<L.grid, (W + 1) * 32, smem, s>>>(L, pol, tmap);
+  kfn<<<L.grid, (W + 2) * 32, smem, s>>>(L, pol, tmap);   // + I/O warp + x-staging warp
   return cudaGetLastError();
 }
 
 template <int K, int W, int D>
 Variant make_nw_variant() {
-  constexpr int U = K >= 8 ? 8 : 16;   // rows per block (TMA box height)
+#ifndef WF_NW_U
+#define WF_NW_U 32
+#endif
+  constexpr int U = K >= 8 ? 16 : WF_NW_U;   // rows per block (TMA box height)
   using S = NwSmem<K, W, D, U>;
-  return Variant{WF_FN_SEQCMP, 0, K, W, D, S::bytes, reinterpret_cast<const void*>(nw_kernel<K, W, D, U, true>),
+  return Variant{WF_FN_SEQCMP, 0, K, W, D, (W + 2) * 32, S::bytes,
+                 reinterpret_cast<const void*>(nw_kernel<K, W, D, U, true>),
                  &launch_nw<K, W, D, U>};
 }
 
@@ -165,7 +170,7 @@ int occupancy(const SweepLaunch& L, int smem) {
     return 0;
   }
   int blocks = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, v->kernel, (v->warps + 1) * 32, smem) != cudaSuccess) {
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, v->kernel, v->threads, smem) != cudaSuccess) {
     cudaGetLastError();
     return 0;
   }

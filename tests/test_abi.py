@@ -82,7 +82,7 @@ def test_local_alignment_is_reported_unsupported():
 
 
 def test_layout_single_slab():
-    lay = query("seqcmp", 1000, lane_cols=4, warps=2, skew=2)
+    lay = query("seqcmp", 1000, lane_cols=4, warps=2, skew=1)
     assert (lay.nplanes, lay.col_begin, lay.col_end) == (1, 0, 1000)
     assert lay.band_cols == 256 and lay.nbands == 4
     assert lay.min_pitch == 1000 and lay.bytes_out == 1000 * 1000 * 4

@@ -43,8 +43,8 @@ def test_seqcmp_dims_default_tiling(dim):
     assert np.array_equal(H, g)
 
 
-SEQ_VARIANTS = [(1, 1, 1), (1, 4, 1), (2, 1, 1), (2, 2, 2), (2, 2, 3), (2, 4, 1), (4, 1, 1), (4, 2, 1), (4, 2, 2),
-                (4, 1, 3), (8, 1, 1), (8, 2, 1)]
+SEQ_VARIANTS = [(1, 1, 1), (1, 4, 1), (2, 1, 1), (2, 2, 2), (2, 2, 3), (2, 4, 1), (4, 1, 1), (4, 2, 1), (4, 1, 2),
+                (4, 1, 3), (8, 1, 1), (8, 1, 2)]
 
 
 @pytest.mark.parametrize("k,w,d", SEQ_VARIANTS)
@@ -115,7 +115,7 @@ def test_seqcmp_determinism_across_tunables():
     dim = 901
     x, y = workloads.seqcmp_inputs(dim, seed_x=5, seed_y=6)
     ref = None
-    for k, w, d in [(1, 1, 1), (2, 2, 3), (4, 2, 2), (8, 1, 2)]:
+    for k, w, d in [(1, 1, 1), (2, 2, 3), (4, 1, 2), (8, 1, 2)]:
         for G in (1, 2):
             (g,) = run_gpu("seqcmp", dim, (x, y), lane_cols=k, warps=w, skew=d, ngpus=G)
             if ref is None:

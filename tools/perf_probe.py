@@ -82,7 +82,12 @@ def main():
                     "ns_per_row_median": float(np.median(steady)),
                     "ns_per_row_band0": float(steady[0]),
                     "sm_ghz_band0": float((tr[0, 43] - tr[0, 42]) / max(1, tr[0, 32] - tr[0, 0])),
-                    "phase_cycles_per_block_band0": [round(float(v) / max(1, dim / 8), 1) for v in tr[0, 44:52]],
+                    "steady_entry_us_first_bands": [[round(float(tr[b, 33 + w] - t0) / 1e3, 2) for w in range(wf.layout.warps)]
+                                                    for b in range(min(6, len(tr)))],
+                    "io_fwd32_feed32_us": [[round(float(tr[b, 36] - t0) / 1e3, 2), round(float(tr[b, 37] - t0) / 1e3, 2)]
+                                           for b in range(min(4, len(tr)))],
+                    "steady_entry_us_band_step": round(float(tr[-1, 33] - tr[0, 33]) / 1e3 / max(1, len(tr) - 1), 2),
+                    "phase_cycles_per_block_band0": [round(float(v) / max(1, dim / 16), 1) for v in tr[0, 48:56]],
                     "feeder_polls": [int(x) for x in tr[:: max(1, len(tr) // 8), 40]],
                     "feeder_empty": [int(x) for x in tr[:: max(1, len(tr) // 8), 41]],
                 })
