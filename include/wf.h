@@ -59,7 +59,8 @@ typedef enum {
   /* Nash-equilibrium stand-in, PAPER.md P:428-431, P:437-439 (dsize = 4):
    * element = 4 int32 (count of pure equilibria, first equilibrium index, its two payoffs)
    * of an n x n bimatrix game (n = tsize) whose payoffs hash the neighbours
-   * (reading R8). */
+   * (reading R8).  Kernel: one warp per column (lane_cols = skew = 1;
+   * warps in {1, 2, 4, 8} = columns per band; default 8). */
   WF_FN_NASH = 1,
   /* Sequence comparison, PAPER.md P:432-435 ("Biological Sequence Comparison [2]"),
    * P:732 ("Smith-Waterman"); Needleman-Wunsch global alignment with linear gap:
@@ -119,7 +120,7 @@ typedef struct {
   int64_t min_pitch;               /* minimum out_pitch in elements (slab columns rounded up to 4) */
   int64_t bytes_out;               /* bytes of all output planes at min_pitch */
   int32_t lane_cols, warps, skew;  /* effective tunables after defaults */
-  int32_t band_cols;               /* columns per CTA band = warps * 32 * lane_cols */
+  int32_t band_cols;               /* columns per CTA band = warps * 32 * lane_cols (NASH: warps) */
   int32_t nbands;                  /* bands in this slab */
   int32_t reserved[5];
 } wf_layout;

@@ -76,6 +76,11 @@ void defaults(const wf_params& p, int* k, int* w, int* d) {
     *k = p.lane_cols ? p.lane_cols : 4;
     *w = p.warps ? p.warps : 2;
     *d = p.skew ? p.skew : 1;
+  } else if (p.fn == WF_FN_NASH) {
+    // one warp per column: lane_cols and skew are fixed at 1
+    *k = p.lane_cols ? p.lane_cols : 1;
+    *w = p.warps ? p.warps : 8;
+    *d = p.skew ? p.skew : 1;
   } else {
     *k = p.lane_cols ? p.lane_cols : 1;
     *w = p.warps ? p.warps : 2;
@@ -129,7 +134,9 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
     case WF_FN_NASH:
       if (p->tsize < 1 || p->tsize > 64) return fail(c, WF_EINVAL, "tsize=%d (strategies) out of range 1..64", p->tsize);
       if (p->dsize != 4) return fail(c, WF_EINVAL, "dsize=%d must be 4 for NASH", p->dsize);
-      return fail(c, WF_EUNSUPPORTED, "fn=NASH kernel not built yet");
+      pl.nf = 4;
+      pl.nbound = 4;
+      break;
     default:
       return fail(c, WF_EINVAL, "fn=%d unknown", p->fn);
   }
@@ -140,7 +147,7 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   if (!wfk::variant_exists(p->fn, p->dsize, pl.k, pl.warps, pl.skew))
     return fail(c, WF_EUNSUPPORTED, "no kernel variant for fn=%d dsize=%d lane_cols=%d warps=%d skew=%d", p->fn,
                 p->dsize, pl.k, pl.warps, pl.skew);
-  pl.band_w = pl.warps * 32 * pl.k;
+  pl.band_w = p->fn == WF_FN_NASH ? pl.warps : pl.warps * 32 * pl.k;   // NASH: one column per warp
   // slabs: every slab but the last is a whole number of bands (its east column is then
   // owned by the last lane of its last band); bands are dealt out as evenly as possible
   const long long B = (cols + pl.band_w - 1) / pl.band_w;

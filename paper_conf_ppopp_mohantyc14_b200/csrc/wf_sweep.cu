@@ -7,6 +7,7 @@
 #include <cudaTypedefs.h>
 
 #include "wf_cells.cuh"
+#include "wf_nash.cuh"
 #include "wf_nw.cuh"
 #include "wf_sweep.cuh"
 
@@ -116,15 +117,41 @@ Variant make_nw_variant() {
                  &launch_nw<K, W, D, U>};
 }
 
+template <int W>
+cudaError_t launch_nash(const SweepLaunch& L, cudaStream_t s, size_t smem) {
+  PolNash pol{};
+  pol.r = static_cast<const uint32_t*>(L.row_in);
+  pol.c = static_cast<const uint32_t*>(L.col_in);
+  for (int p = 0; p < 4; ++p) {
+    pol.topp[p] = static_cast<const int32_t*>(L.top[p]);
+    pol.leftp[p] = static_cast<const int32_t*>(L.left[p]);
+  }
+  auto kfn = L.tsize == 16 ? nash_kernel<W, 16> : nash_kernel<W, 0>;   // n = 16: register fast path
+  cudaError_t e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  if (e != cudaSuccess) return e;
+  kfn<<<L.grid, (W + 1) * 32, smem, s>>>(L, pol);
+  return cudaGetLastError();
+}
+
+// NASH: one warp per column (lane_cols = 1, skew = 1); smem listed without the per-warp
+// game scratch, which depends on n (added by smem_bytes()).
+template <int W>
+Variant make_nash_variant() {
+  return Variant{WF_FN_NASH, 0, 1, W, 1, (W + 1) * 32, NashSmem<W>::fixed_bytes,
+                 reinterpret_cast<const void*>(nash_kernel<W, 16>), &launch_nash<W>};
+}
+
 // --- the compiled variant set -------------------------------------------------------
 #define WF_SEQ(K, W, D) make_nw_variant<K, W, D>()
 #define WF_SYN(DS, K, W, D) make_variant<PolSyn<DS>, K, W, D>(WF_FN_SYNTHETIC, DS)
+#define WF_NASH(W) make_nash_variant<W>()
 #define WF_SYN_DS(DS) WF_SYN(DS, 1, 1, 1), WF_SYN(DS, 1, 2, 1), WF_SYN(DS, 1, 4, 1), WF_SYN(DS, 2, 1, 1), \
     WF_SYN(DS, 2, 2, 1), WF_SYN(DS, 1, 2, 2), WF_SYN(DS, 2, 2, 2)
 
 const Variant* table(size_t* n) {
 #ifdef WF_MIN_VARIANTS   // quick experimental builds (tools/ablate.sh)
-  static const Variant v[] = {WF_SEQ(4, 1, 1), WF_SEQ(4, 1, 2), WF_SEQ(4, 2, 1), WF_SEQ(2, 1, 1), WF_SEQ(8, 1, 1)};
+  static const Variant v[] = {WF_SEQ(4, 1, 1), WF_SEQ(4, 1, 2), WF_SEQ(4, 2, 1), WF_SEQ(2, 1, 1), WF_SEQ(8, 1, 1),
+                              WF_NASH(8)};
 #else
   static const Variant v[] = {
       WF_SEQ(2, 1, 1), WF_SEQ(2, 2, 1), WF_SEQ(2, 4, 1), WF_SEQ(2, 1, 2), WF_SEQ(2, 2, 2), WF_SEQ(2, 4, 2),
@@ -135,6 +162,7 @@ const Variant* table(size_t* n) {
       WF_SEQ(1, 1, 1), WF_SEQ(1, 2, 1), WF_SEQ(1, 4, 1),
       WF_SYN_DS(0), WF_SYN_DS(1), WF_SYN_DS(2), WF_SYN_DS(3), WF_SYN_DS(4),
       WF_SYN_DS(5), WF_SYN_DS(6), WF_SYN_DS(7), WF_SYN_DS(8),
+      WF_NASH(1), WF_NASH(2), WF_NASH(4), WF_NASH(8),
   };
 #endif
   *n = sizeof(v) / sizeof(v[0]);
@@ -159,7 +187,9 @@ bool variant_exists(int fn, int dsize, int k, int warps, int skew) {
 
 int smem_bytes(const SweepLaunch& L) {
   const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : 0, L.k, L.warps, L.skew);
-  return v ? (int)v->smem : -1;
+  if (!v) return -1;
+  if (L.fn == WF_FN_NASH) return (int)(v->smem + size_t(L.warps) * ((size_t(2) * L.tsize * L.tsize + 2 * L.tsize + 15) & ~size_t(15)));
+  return (int)v->smem;
 }
 
 int occupancy(const SweepLaunch& L, int smem) {
@@ -180,7 +210,7 @@ int occupancy(const SweepLaunch& L, int smem) {
 cudaError_t launch(const SweepLaunch& L, cudaStream_t s) {
   const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : 0, L.k, L.warps, L.skew);
   if (!v) return cudaErrorInvalidDeviceFunction;
-  return v->launch(L, s, v->smem);
+  return v->launch(L, s, (size_t)smem_bytes(L));
 }
 
 int variant_count() {

@@ -105,6 +105,7 @@ struct Watchdog {
 // Shared-memory carve-up for one CTA.
 template <int NF, int K, int WARPS, int D>
 struct Smem {
+  static constexpr int kSlots = kHandSlots;
   static constexpr int R = ring_rows(D);
   static constexpr size_t stage_words = size_t(WARPS) * NF * R * 32 * K;     // u32
   static constexpr size_t hand_words = size_t(WARPS) * kHandSlots * NF;       // u64
@@ -138,11 +139,11 @@ __device__ __forceinline__ bool feeder(const SweepLaunch& L, const P& pol, const
   Watchdog wd;
   wd.start();
   while (base <= L.rows) {
-    // back-pressure: rows base .. base+63 go to slots that held rows base-256 .. ;
+    // back-pressure: rows base .. base+63 go to slots that held rows base-kSlots .. ;
     // those must have been consumed by compute warp 0.
     // The feeder is normally far ahead, so it sleeps between polls: a tight LDS spin would
     // occupy the SM's MIO pipe that the compute warps' SHFL/LDS/STS depend on.
-    const int need = base + 63 - kHandSlots;
+    const int need = base + 63 - SM::kSlots;
     while (seen_prog < need) {
       seen_prog = lds_vol_i(sm.prog + 0);
       if (seen_prog < need) {

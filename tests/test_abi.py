@@ -103,6 +103,27 @@ def test_layout_slabs_partition_columns(dim, G):
     assert sum(l.width for l in lays) == dim
 
 
+def test_nash_layout_one_column_per_warp():
+    lay = query("nash", 4096, tsize=16, dsize=4)
+    assert lay.nplanes == 4 and lay.nbound == 4 and lay.plane_is_float == [False] * 4
+    assert (lay.lane_cols, lay.warps, lay.skew) == (1, 8, 1)
+    assert lay.band_cols == 8 and lay.nbands == 512
+    lays = [query("nash", 4096, tsize=16, dsize=4, ngpus=2, rank=g) for g in range(2)]
+    assert lays[0].col_end == lays[1].col_begin == 2048
+
+
+@pytest.mark.parametrize("kw,field", [(dict(tsize=0, dsize=4), "tsize"), (dict(tsize=65, dsize=4), "tsize"),
+                                      (dict(tsize=16, dsize=3), "dsize")])
+def test_nash_rejects_bad_params(kw, field):
+    e = _err("nash", 100, **kw)
+    assert e.status == _abi.WF_EINVAL and field in str(e)
+
+
+def test_nash_rejects_multi_column_lanes():
+    e = _err("nash", 100, tsize=16, dsize=4, lane_cols=2)
+    assert e.status == _abi.WF_EUNSUPPORTED
+
+
 def test_slab_count_too_large_is_rejected():
     e = _err("seqcmp", 300, ngpus=4, rank=0, lane_cols=4, warps=2)
     assert e.status == _abi.WF_EINVAL and "empty" in str(e)

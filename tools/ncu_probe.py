@@ -17,11 +17,15 @@ dev = torch.device("cuda", 0)
 t = lambda a: torch.from_numpy(np.ascontiguousarray(a)).to(dev)
 if fn == "seqcmp":
     x, y = workloads.seqcmp_inputs(dim, cols or dim); ins = (t(x), t(y), None, None); kw = {}
+elif fn == "nash":
+    r, c, top, left = workloads.nash_inputs(dim, cols or dim)
+    ins = (t(r), t(c), [t(top[i]) for i in range(4)], [t(left[i]) for i in range(4)])
+    kw = dict(tsize=tsize or 16, dsize=4)
 else:
     u, v, top, left = workloads.synthetic_inputs(dim, cols or dim, dsize)
     ins = (t(u), t(v), [t(top[i]) for i in range(dsize)], [t(left[i]) for i in range(dsize)])
     kw = dict(tsize=tsize, dsize=dsize)
-wf = Wavefront(fn, dim, cols=cols, lane_cols=k, warps=w, skew=d, **({"alphabet": 4} if fn == "seqcmp" else {}), **kw)
+wf = Wavefront(fn, dim, cols=cols, lane_cols=k, warps=w, skew=d, watchdog_cycles=1 << 42, **({"alphabet": 4} if fn == "seqcmp" else {}), **kw)
 out = wf.alloc_out()
 for _ in range(reps):
     wf.run(*ins, out=out)

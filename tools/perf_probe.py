@@ -24,6 +24,9 @@ def inputs(fn, dim, dsize, dev, cols=0):
     if fn == "seqcmp":
         x, y = workloads.seqcmp_inputs(dim, cols or dim)
         return t(x), t(y), None, None
+    if fn == "nash":
+        r, c, top, left = workloads.nash_inputs(dim, cols or dim)
+        return t(r), t(c), [t(top[p]) for p in range(4)], [t(left[p]) for p in range(4)]
     u, v, top, left = workloads.synthetic_inputs(dim, cols or dim, dsize)
     return t(u), t(v), [t(top[d]) for d in range(dsize)], [t(left[d]) for d in range(dsize)]
 
@@ -50,6 +53,8 @@ def main():
                 kw.update(alphabet=a.alphabet)
             if a.fn == "synthetic":
                 kw.update(tsize=a.tsize, dsize=a.dsize)
+            if a.fn == "nash":
+                kw.update(tsize=a.tsize or 16, dsize=4)
             try:
                 wf = Wavefront(a.fn, dim, cols=a.cols, **kw)
             except Exception as e:  # noqa: BLE001
