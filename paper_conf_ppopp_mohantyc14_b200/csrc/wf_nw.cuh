@@ -152,8 +152,14 @@ struct NwWarp {
     gap = L.gap;
     mmatch = L.match;
     mmis = L.mismatch;
+#ifndef WF_NW_OPAQUE_GK
+#define WF_NW_OPAQUE_GK 0
+#endif
 #pragma unroll
-    for (int m = 0; m < K; ++m) gk[m] = (m + 1) * gap;
+    for (int m = 0; m < K; ++m) {
+      gk[m] = (m + 1) * gap;
+      if (WF_NW_OPAQUE_GK) asm volatile("mov.b32 %0, %0;" : "+r"(gk[m]));   // keep W + gk[m] a DPX add-max
+    }
     const uint8_t* y = static_cast<const uint8_t*>(L.col_in);
     wcol = band * L.band_w + warp * 32 * K;
     const int jb = L.c0 + wcol + lane * K;    // global 0-based column of the lane's first column
@@ -274,8 +280,86 @@ struct NwWarp {
     }
   }
 
+#ifndef WF_NW_ROT
+#define WF_NW_ROT 0
+#endif
+  // Rotation form (D = 1): lane 31 hands lane 0 its next west input and row code through the
+  // same lane-rotating shuffle that carries every other lane's east value, so the only
+  // instructions on the lane-to-lane chain are SHFL and one VIADDMNMX:
+  //   src = max(W + gL, PL), gL = K*g, PL = P_{K-1} (lanes 0..30)  -> H[K-1]
+  //                          gL = -2^28, PL = w0 of the next row (lane 31) -> w0'
+  template <bool EDGE>
+  __device__ __forceinline__ void block_rot(int t0, int32_t wv, uint32_t xv, int32_t& east_last) {
+    const int src_lane = (lane + 31) & 31;
+    int32_t gL;
+    asm volatile("mov.b32 %0, %1;" : "=r"(gL) : "r"(lane == 31 ? -(1 << 28) : K * gap));
+    const int32_t w00 = __shfl_sync(0xffffffffu, wv, 0);    // shuffles outside the selects:
+    const uint32_t x00 = __shfl_sync(0xffffffffu, xv, 0);   // every lane must execute them
+    int32_t Win = (lane == 0) ? w00 : q[0];
+    uint32_t Xin = (lane == 0) ? x00 : xq[0];
+#pragma unroll
+#ifndef WF_NW_ABL
+#define WF_NW_ABL 0   // performance archaeology only (wrong grids): 1 no STS, 2 no x shuffles, 4 no w0 shuffle
+#endif
+    for (int u = 0; u < U; ++u) {
+      const int row = t0 + u - lane + 1;
+      const int32_t w0n = (WF_NW_ABL & 4) ? u : __shfl_sync(0xffffffffu, wv, (u + 1) & (U - 1));   // next row of lane 0
+      const uint32_t x0n = (WF_NW_ABL & 2) ? 1u : __shfl_sync(0xffffffffu, xv, (u + 1) & (U - 1));
+      int32_t H[K];
+      int32_t Pl;
+      cells_p(Win, Xin, H, Pl);
+      const int32_t PL = (lane == 31) ? w0n : Pl;
+      const int32_t src = __viaddmax_s32(Win, gL, PL);
+      const uint32_t xsrc = (lane == 31) ? x0n : Xin;
+      if constexpr ((WF_NW_ABL & 1) != 0) {
+        prevW = Win;
+#pragma unroll
+        for (int m = 0; m < K; ++m) Np[m] = H[m];
+        if (u == U - 1) stage_store(row, H);
+      } else if constexpr (EDGE) {
+        const bool active = row >= 1 && row <= rows;
+        prevW = active ? Win : prevW;
+#pragma unroll
+        for (int m = 0; m < K; ++m) Np[m] = active ? H[m] : Np[m];
+        if (active) stage_store(row, H);
+      } else {
+        prevW = Win;
+#pragma unroll
+        for (int m = 0; m < K; ++m) Np[m] = H[m];
+        stage_store(row, H);
+      }
+      Win = __shfl_sync(0xffffffffu, src, src_lane);
+      if constexpr ((WF_NW_ABL & 2) == 0) Xin = __shfl_sync(0xffffffffu, xsrc, src_lane);
+    }
+    // lanes 1..31 carry their next west input into the next block in q[0]
+    q[0] = Win;
+    xq[0] = Xin;
+    east_last = Np[K - 1];
+  }
+
+  // prefix cells returning P_{K-1} as well (the rotation form recomputes H[K-1] for lane 31)
+  __device__ __forceinline__ void cells_p(int32_t Win, uint32_t xc, int32_t (&H)[K], int32_t& Plast) const {
+    const uint32_t sel = xc * 0x1111u + 0x8880u;
+    int32_t P = 0;
+#pragma unroll
+    for (int m = 0; m < K; ++m) {
+      const int32_t NW = m == 0 ? prevW : Np[m - 1];
+      int32_t s;
+      if constexpr (PRMT) s = prmt_s8(qlo[m], qhi[m], sel);
+      else s = (xc == ycode[m]) ? mmatch : mmis;
+      const int32_t t1 = __viaddmax_s32(Np[m], gap, NW + s);
+      P = (m == 0) ? t1 : __viaddmax_s32(P, gap, t1);
+      H[m] = __viaddmax_s32(Win, gk[m], P);
+    }
+    Plast = P;
+  }
+
   template <bool EDGE>
   __device__ __forceinline__ void block(int t0, int32_t wv, uint32_t xv, int32_t& east_last) {
+    if constexpr (WF_NW_ROT != 0 && D == 1) {
+      block_rot<EDGE>(t0, wv, xv, east_last);
+      return;
+    }
 #pragma unroll
     for (int u = 0; u < U; ++u) {
       const int row = t0 + u - D * lane + 1;
@@ -323,6 +407,18 @@ struct NwWarp {
       L.trace[size_t(band) * kTraceSlots + 42] = clock64();
     }
     int blk = 0;
+    // WF_TRACE phase profile (lane 0 of warps 0..2): SM cycles spent per block phase --
+    // [0] west wait, [1] west loads, [2] free-slot wait, [3] row compute, [4] publish
+    const bool prof = L.trace != nullptr && lane == 0 && warp < 3;
+    long long ph[5] = {0, 0, 0, 0, 0};
+    long long tc = prof ? clock64() : 0;
+    auto tick = [&](int i) {
+      if (prof) {
+        const long long n = clock64();
+        ph[i] += n - tc;
+        tc = n;
+      }
+    };
     for (; t0 < T; t0 += U, ++blk) {
       const int r0 = t0 + 1;                       // lane 0's first row in this block
       const int rl = min(t0 + U, rows);            // its last valid row
@@ -332,6 +428,7 @@ struct NwWarp {
       if (rl >= 1) {
         if (!wait_ctr(wprog_src, rl, seen_wprog, 20)) return false;
         if (!wait_ctr(sm.xfill, rl, seen_xfill, 32)) return false;
+        tick(0);
         const int r = r0 + lane;
         if (lane < U && r >= 1 && r <= rows) {
           wv = lds_vol_s32(wsrc + ((r + wsrc_off) & wmask) * wstride);
@@ -344,6 +441,7 @@ struct NwWarp {
         sts_vol_i(rprog_src, r0 - U - 1 + U);
         sts_vol_i(sm.xneed + warp, r0);
       }
+      tick(1);
       // ---- my staging ring: slots of rows <= lane 0's rows of this block minus R must be
       //      free: read by TMA (bulk groups) and by my reader (rprog[warp])
       const int need_free = t0 + U - R;
@@ -352,12 +450,14 @@ struct NwWarp {
         __syncwarp();
         if (!wait_ctr(sm.rprog + warp, need_free, seen_rprog, 20)) return false;
       }
+      tick(2);
       int32_t east_last;
       if (L.trace && lane == 0 && t0 <= steady_lo && t0 + U > steady_lo)   // entering steady state
         L.trace[size_t(band) * kTraceSlots + 33 + warp] = globaltimer();
       if (t0 >= steady_lo && t0 <= steady_hi) block<false>(t0, wv, xv, east_last);
       else block<true>(t0, wv, xv, east_last);
       (void)east_last;
+      tick(3);
       // ---- publish: one fence for the TMA engine and for the next warp
       const int r31_0 = t0 - 31 * D + 1;           // first row of the block's TMA box
       const int r31_last = min(r31_0 + U - 1, rows);
@@ -374,7 +474,10 @@ struct NwWarp {
         }
         if (lane == 0) sts_vol_i(sm.wprog + warp, r31_last);
       }
+      tick(4);
     }
+    if (prof)
+      for (int i = 0; i < 5; ++i) L.trace[size_t(band) * kTraceSlots + 48 + 5 * warp + i] = ph[i];
     if (lane == 0) {
       bulk_wait_all();
       sts_vol_i(rprog_src, rows);

@@ -92,7 +92,13 @@ def main():
                     "io_fwd32_feed32_us": [[round(float(tr[b, 36] - t0) / 1e3, 2), round(float(tr[b, 37] - t0) / 1e3, 2)]
                                            for b in range(min(4, len(tr)))],
                     "steady_entry_us_band_step": round(float(tr[-1, 33] - tr[0, 33]) / 1e3 / max(1, len(tr) - 1), 2),
-                    "phase_cycles_per_block_band0": [round(float(v) / max(1, dim / 16), 1) for v in tr[0, 48:56]],
+                    # NW: per warp (lane 0) SM cycles per row step in [west wait, west loads,
+                    # free wait, compute, publish]; band 0 and the middle band
+                    "nw_phase_cyc_per_row_band0": [[round(float(v) / dim, 1) for v in tr[0, 48 + 5 * w:53 + 5 * w]]
+                                                   for w in range(min(3, wf.layout.warps))],
+                    "nw_phase_cyc_per_row_mid": [[round(float(v) / dim, 1)
+                                                  for v in tr[len(tr) // 2, 48 + 5 * w:53 + 5 * w]]
+                                                 for w in range(min(3, wf.layout.warps))],
                     "feeder_polls": [int(x) for x in tr[:: max(1, len(tr) // 8), 40]],
                     "feeder_empty": [int(x) for x in tr[:: max(1, len(tr) // 8), 41]],
                 })
