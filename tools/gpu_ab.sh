@@ -14,5 +14,6 @@ for l in open(f"gpurun_out/ab_{sys.argv[1]}.log"):
     print(d.get("variant"), d.get("ms"), d.get("gcups"), "band_end", d.get("band_end_us", [])[:1], d.get("band_end_us", [])[-1:])
     print("  steady_entry", d.get("steady_entry_us_first_bands", [])[:3], "io", d.get("io_fwd32_feed32_us"))
     print("  ph0", d.get("nw_phase_cyc_per_row_band0"), "mid", d.get("nw_phase_cyc_per_row_mid"))
+    print("  slow", d.get("nw_slow_west_entries_polls_band0"), d.get("nw_slow_west_entries_polls_mid"))
 PY
 done

@@ -94,11 +94,15 @@ def main():
                     "steady_entry_us_band_step": round(float(tr[-1, 33] - tr[0, 33]) / 1e3 / max(1, len(tr) - 1), 2),
                     # NW: per warp (lane 0) SM cycles per row step in [west wait, west loads,
                     # free wait, compute, publish]; band 0 and the middle band
-                    "nw_phase_cyc_per_row_band0": [[round(float(v) / dim, 1) for v in tr[0, 48 + 5 * w:53 + 5 * w]]
-                                                   for w in range(min(3, wf.layout.warps))],
+                    "nw_phase_cyc_per_row_band0": [[round(float(v) / dim, 1) for v in tr[0, 48 + 4 * w:52 + 4 * w]]
+                                                   for w in range(min(4, wf.layout.warps))],
                     "nw_phase_cyc_per_row_mid": [[round(float(v) / dim, 1)
-                                                  for v in tr[len(tr) // 2, 48 + 5 * w:53 + 5 * w]]
-                                                 for w in range(min(3, wf.layout.warps))],
+                                                  for v in tr[len(tr) // 2, 48 + 4 * w:52 + 4 * w]]
+                                                 for w in range(min(4, wf.layout.warps))],
+                    "nw_slow_west_entries_polls_band0": [int(tr[0, 43 + w])
+                                                         for w in range(min(4, wf.layout.warps))],
+                    "nw_slow_west_entries_polls_mid": [int(tr[len(tr) // 2, 43 + w])
+                                                        for w in range(min(4, wf.layout.warps))],
                     "feeder_polls": [int(x) for x in tr[:: max(1, len(tr) // 8), 40]],
                     "feeder_empty": [int(x) for x in tr[:: max(1, len(tr) // 8), 41]],
                 })
