@@ -1,5 +1,6 @@
 // wf_sweep.cu -- instantiations and host-side launch of the persistent band sweep.
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <type_traits>
 
@@ -10,6 +11,7 @@
 #include "wf_nash.cuh"
 #include "wf_nw.cuh"
 #include "wf_sweep.cuh"
+#include "wf_variant.h"
 
 namespace wfk {
 
@@ -23,14 +25,6 @@ int nwords(int fn, int dsize) {
 }
 
 namespace {
-
-struct Variant {
-  int fn, dsize, k, warps, skew;
-  int threads;         // CTA size (compute warps + helper warps)
-  size_t smem;
-  const void* kernel;  // __global__ function pointer (for occupancy queries)
-  cudaError_t (*launch)(const SweepLaunch&, cudaStream_t, size_t);
-};
 
 template <class P, int K, int W, int D>
 cudaError_t launch_t(const SweepLaunch& L, cudaStream_t s, size_t smem) {
@@ -61,8 +55,10 @@ template <class P, int K, int W, int D>
 Variant make_variant(int fn, int dsize) {
   using S = Smem<P::NF, K, W, D>;
   return Variant{fn, dsize, K, W, D, (W + 1) * 32, S::bytes, reinterpret_cast<const void*>(sweep_kernel<P, K, W, D>),
-                 &launch_t<P, K, W, D>};
+                 &launch_t<P, K, W, D>, 4};
 }
+
+}  // namespace
 
 // cuTensorMapEncodeTiled through the runtime's driver entry point (no -lcuda link needed)
 cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols, int box_rows) {
@@ -83,6 +79,8 @@ cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols,
                    CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   return r == CUDA_SUCCESS ? cudaSuccess : cudaErrorInvalidValue;
 }
+
+namespace {
 
 template <int K, int W, int D, int U>
 cudaError_t launch_nw(const SweepLaunch& L, cudaStream_t s, size_t smem) {
@@ -114,7 +112,7 @@ Variant make_nw_variant() {
   using S = NwSmem<K, W, D, U>;
   return Variant{WF_FN_SEQCMP, 0, K, W, D, (W + 2) * 32, S::bytes,
                  reinterpret_cast<const void*>(nw_kernel<K, W, D, U, true>),
-                 &launch_nw<K, W, D, U>};
+                 &launch_nw<K, W, D, U>, 4};
 }
 
 template <int W>
@@ -138,7 +136,7 @@ cudaError_t launch_nash(const SweepLaunch& L, cudaStream_t s, size_t smem) {
 template <int W>
 Variant make_nash_variant() {
   return Variant{WF_FN_NASH, 0, 1, W, 1, (W + 1) * 32, NashSmem<W>::fixed_bytes,
-                 reinterpret_cast<const void*>(nash_kernel<W, 16>), &launch_nash<W>};
+                 reinterpret_cast<const void*>(nash_kernel<W, 16>), &launch_nash<W>, 4};
 }
 
 // --- the compiled variant set -------------------------------------------------------
@@ -169,8 +167,20 @@ const Variant* table(size_t* n) {
   return v;
 }
 
+// SEQCMP at skew 1: the v4 kernel (block hand-offs) is the default -- measured faster on C4
+// (profiles/r01_nw7_experiments.txt); WF_NW_IMPL=7 selects the per-row hand-off v7 kernel
+bool want_nw7() {
+  const char* e = getenv("WF_NW_IMPL");
+  return e && e[0] == '7';
+}
+
 const Variant* find(int fn, int dsize, int k, int warps, int skew) {
   size_t n;
+  if (fn == WF_FN_SEQCMP && skew == 1 && want_nw7()) {
+    const Variant* t7 = nw7_table(&n);
+    for (size_t i = 0; i < n; ++i)
+      if (t7[i].k == k && t7[i].warps == warps) return &t7[i];
+  }
   const Variant* t = table(&n);
   for (size_t i = 0; i < n; ++i)
     if (t[i].fn == fn && t[i].dsize == dsize && t[i].k == k && t[i].warps == warps && t[i].skew == skew) return &t[i];

@@ -1,0 +1,22 @@
+// wf_variant.h -- the compiled kernel-variant table entry (host side, not part of the ABI).
+#pragma once
+#include <cstddef>
+#include <cuda_runtime.h>
+
+#include "wf_internal.h"
+
+namespace wfk {
+
+struct Variant {
+  int fn, dsize, k, warps, skew;
+  int threads;         // CTA size (compute warps + helper warps)
+  size_t smem;
+  const void* kernel;  // __global__ function pointer (for occupancy queries)
+  cudaError_t (*launch)(const SweepLaunch&, cudaStream_t, size_t);
+  int impl;            // kernel generation (SEQCMP: 4 = block hand-offs, 7 = per-row hand-offs)
+};
+
+// SEQCMP v7 variants (wf_nw7.cu)
+const Variant* nw7_table(size_t* n);
+
+}  // namespace wfk

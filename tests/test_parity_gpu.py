@@ -55,6 +55,25 @@ def test_seqcmp_variants(k, w, d, dim, alphabet):
     assert np.array_equal(H, g)
 
 
+@pytest.mark.parametrize("form", ["0", "1"])
+@pytest.mark.parametrize("k,w", [(4, 1), (4, 2), (2, 2), (2, 4), (8, 1)])
+@pytest.mark.parametrize("dim", [1, 33, 64, 97, 777, 1100])
+@pytest.mark.parametrize("alphabet", [0, 4])
+def test_seqcmp_v7_kernel(monkeypatch, form, k, w, dim, alphabet):
+    """The per-row hand-off kernel (wf_nw7.cu, opt-in via WF_NW_IMPL=7) against the oracle."""
+    monkeypatch.setenv("WF_NW_IMPL", "7")
+    monkeypatch.setenv("WF_NW7_FORM", form)
+    H, g = _seq(dim, lane_cols=k, warps=w, skew=1, seed=(dim + 5, dim + 6), alphabet=alphabet)
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.parametrize("G", [2, 3])
+def test_seqcmp_v7_local_slabs(monkeypatch, G):
+    monkeypatch.setenv("WF_NW_IMPL", "7")
+    H, g = _seq(1000, lane_cols=4, warps=2, skew=1, ngpus=G, alphabet=4)
+    assert np.array_equal(H, g)
+
+
 @pytest.mark.parametrize("alphabet", [4, 8])
 @pytest.mark.parametrize("scoring", [(1, -1, -1), (2, -3, -1), (-3, 2, -1), (64, -64, -64), (-64, 64, 64)])
 def test_seqcmp_byte_permute_scores(alphabet, scoring):

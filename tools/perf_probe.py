@@ -105,6 +105,8 @@ def main():
                                                         for w in range(min(4, wf.layout.warps))],
                     "feeder_polls": [int(x) for x in tr[:: max(1, len(tr) // 8), 40]],
                     "feeder_empty": [int(x) for x in tr[:: max(1, len(tr) // 8), 41]],
+                    "raw32_band0": [int(x) for x in tr[0, 32:64]],
+                    "raw32_mid": [int(x) for x in tr[len(tr) // 2, 32:64]],
                 })
             print(json.dumps(rec))
             res.append(rec)

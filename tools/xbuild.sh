@@ -8,7 +8,8 @@ mkdir -p /tmp/wfx tools/abl_out
 N=/usr/local/cuda/bin/nvcc
 F="-gencode arch=compute_100a,code=sm_100a -O3 -lineinfo -std=c++17 -Xcompiler -fPIC --expt-relaxed-constexpr -Iinclude -Ipaper_conf_ppopp_mohantyc14_b200/csrc -DWF_MIN_VARIANTS"
 $N $F "$@" -c paper_conf_ppopp_mohantyc14_b200/csrc/wf_api.cpp -o /tmp/wfx/api_$NAME.o &
+$N $F "$@" -c paper_conf_ppopp_mohantyc14_b200/csrc/wf_nw7.cu -o /tmp/wfx/nw7_$NAME.o &
 $N $F "$@" -c paper_conf_ppopp_mohantyc14_b200/csrc/wf_sweep.cu -o /tmp/wfx/sweep_$NAME.o
 wait
-$N -gencode arch=compute_100a,code=sm_100a -shared -cudart static -o tools/abl_out/libwf_$NAME.so /tmp/wfx/sweep_$NAME.o /tmp/wfx/api_$NAME.o
+$N -gencode arch=compute_100a,code=sm_100a -shared -cudart static -o tools/abl_out/libwf_$NAME.so /tmp/wfx/sweep_$NAME.o /tmp/wfx/nw7_$NAME.o /tmp/wfx/api_$NAME.o
 echo tools/abl_out/libwf_$NAME.so
