@@ -47,6 +47,65 @@ def load_peaks():
         return 6650.0, "fallback (B200_PROFILING.md 6.65 TB/s)"
 
 
+SMS = 148
+FP32_LANES_PER_SM = 128      # B200_PROFILING.md unit counts: 4 SMSPs x 32 FP32 lanes
+CELL_CHAIN_CYC = 4.12        # dependent FADD/FMUL/FFMA latency, profiles/r01_microbench.txt (lat_ffma_cyc)
+NASH_INT_OPS_PER_CELL = 5120  # n=16: 2 n^2 payoff hashes x ~8 int ops + n^2 best-response tests x ~4
+
+
+def roofline_model(cfg, slab_cells, avg_launch_ms, world):
+    """The dominant kernel's roof for this config.
+
+    seqcmp and low-tsize synthetic: HBM, algorithmic bytes = cells x B/cell (each output cell
+    written once).  High-tsize synthetic and Nash: plain FP32 / INT32 ALU issue, algorithmic
+    ops = cells x ops/cell.  The bound is the slower roof; both are reported, plus the
+    dependency-chain (latency) roof of the 2*dim-1 anti-diagonals as a diagnostic."""
+    hbm_peak, hbm_src = load_peaks()
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            mhz = float(json.load(f).get("sm_max_mhz", 1965.0))
+    except Exception:
+        mhz = 1965.0
+    ghz = mhz / 1e3
+    secs = avg_launch_ms * 1e-3
+    bpc = cfg.bytes_per_cell()
+    hbm = {"achieved": slab_cells * bpc / secs / 1e9, "peak": hbm_peak, "unit": "GB/s",
+           "roof_gcups": hbm_peak / bpc, "algorithmic_bytes_per_launch": slab_cells * bpc, "peak_source": hbm_src}
+    if cfg.fn == "seqcmp":
+        alu = None
+    else:
+        if cfg.fn == "synthetic":
+            ops = 2 + cfg.dsize * (cfg.tsize + 3)   # c = (u*v)*2^-12; per item 2 FADD + FMUL + tsize FFMA
+            chain = CELL_CHAIN_CYC * (cfg.tsize + 3) if cfg.dsize else CELL_CHAIN_CYC
+            kind = "FP32"
+        else:
+            ops = NASH_INT_OPS_PER_CELL
+            chain = None
+            kind = "INT32"
+        peak_ops = SMS * FP32_LANES_PER_SM * ghz   # G lane-ops/s
+        alu = {"achieved": slab_cells * ops / secs / 1e9, "peak": peak_ops, "unit": f"G{kind} op/s",
+               "ops_per_cell": ops, "roof_gcups": peak_ops / ops,
+               "peak_source": f"{SMS} SMs x {FP32_LANES_PER_SM} lanes x {mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)"}
+    if alu is not None and alu["roof_gcups"] < hbm["roof_gcups"]:
+        dom, bound = alu, "alu"
+    else:
+        dom, bound = hbm, "hbm"
+    out = {"bound": bound, "achieved": dom["achieved"], "peak": dom["peak"], "unit": dom["unit"],
+           "frac": dom["achieved"] / dom["peak"], "peak_source": dom["peak_source"], "avg_launch_ms": avg_launch_ms,
+           "roof_gcups_per_gpu": dom["roof_gcups"], "hbm": hbm}
+    if alu is not None:
+        out["alu"] = alu
+    if cfg.fn == "synthetic" and cfg.dsize:
+        diag = 2 * cfg.dim - 1
+        lat_gcups = cfg.dim * cfg.dim / (diag * chain / (ghz * 1e9)) / 1e9
+        out["latency_roof"] = {"gcups": lat_gcups, "cycles_per_cell_on_chain": chain, "anti_diagonals": diag,
+                               "note": "dependency chain: every anti-diagonal needs one full cell (tsize-deep "
+                                       "FMA chain) after its predecessor; no schedule can beat it"}
+    if bound == "hbm":
+        out["algorithmic_bytes_per_launch"] = hbm["algorithmic_bytes_per_launch"]
+    return out
+
+
 def load_traffic(workload_key):
     try:
         with open(os.path.join(ROOT, "profiles", "ncu_traffic.json")) as f:
@@ -329,11 +388,10 @@ def run_ours(args, cfg):
                     "d2h_bytes_per_step": int(footprint), "h2d_bytes_per_step": h2d}
         del host_grid
 
-    peak, peak_src = load_peaks()
-    bytes_per_launch = slab_cells * cfg.bytes_per_cell()
-    achieved = bytes_per_launch / (avg_launch_ms * 1e-3) / 1e9
+    roof = roofline_model(cfg, slab_cells, avg_launch_ms, world)
     key = f"{cfg.name}_k{lay.lane_cols}w{lay.warps}d{lay.skew}"
-    traffic = load_traffic(key)
+    roof["traffic"] = load_traffic(key)
+    roof["kernel"] = {"seqcmp": "wfk::nw_kernel", "synthetic": "wfk::syn_kernel", "nash": "wfk::nash_kernel"}[cfg.fn]
 
     result = None
     if rank == 0:
@@ -348,10 +406,7 @@ def run_ours(args, cfg):
                        "l2": ("explicit 252 MiB L2 flush between steps (footprint < 2x L2)" if flush else
                               f"outputs {footprint / 2**30:.2f} GiB per GPU > 126 MB L2; no flush needed")},
             "gpu_launches": args.steps * world,
-            "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
-                         "traffic": traffic, "peak_source": peak_src,
-                         "algorithmic_bytes_per_launch": bytes_per_launch, "avg_launch_ms": avg_launch_ms,
-                         "kernel": "wfk::nw_kernel" if cfg.fn == "seqcmp" else "wfk::sweep_kernel"},
+            "roofline": roof,
             "e2e": {"value": total_cells / (e2e_ms * 1e-3) / 1e9, "unit": UNIT, "ms_per_step": e2e_ms,
                     "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                     "note": "H2D of the step's inputs from pinned memory, sweep, D2H of the result row"},

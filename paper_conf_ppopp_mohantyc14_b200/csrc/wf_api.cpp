@@ -77,13 +77,17 @@ void defaults(const wf_params& p, int* k, int* w, int* d) {
     *w = p.warps ? p.warps : 2;
     *d = p.skew ? p.skew : 1;
   } else if (p.fn == WF_FN_NASH) {
-    // one warp per column: lane_cols and skew are fixed at 1
-    *k = p.lane_cols ? p.lane_cols : 1;
-    *w = p.warps ? p.warps : 8;
-    *d = p.skew ? p.skew : 1;
-  } else {
+    // one warp per column: lane_cols and skew are fixed at 1; 2 columns per CTA measured
+    // fastest on C3 (profiles/autotune_C3.json)
     *k = p.lane_cols ? p.lane_cols : 1;
     *w = p.warps ? p.warps : 2;
+    *d = p.skew ? p.skew : 1;
+  } else {
+    // synthetic (wf_syn.cu): one column per lane keeps the tsize-deep FMA chain per step
+    // short; one compute warp per CTA (32-column bands, several CTAs per SM share its
+    // SMSPs) measured fastest on C5a/C5b (tools/autotune.py, profiles/autotune_*.json)
+    *k = p.lane_cols ? p.lane_cols : 1;
+    *w = p.warps ? p.warps : 1;
     *d = p.skew ? p.skew : 1;
   }
 }

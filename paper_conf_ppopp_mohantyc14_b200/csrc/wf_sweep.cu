@@ -61,7 +61,7 @@ Variant make_variant(int fn, int dsize) {
 }  // namespace
 
 // cuTensorMapEncodeTiled through the runtime's driver entry point (no -lcuda link needed)
-cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols, int box_rows) {
+cudaError_t encode_plane_map_f(CUtensorMap* m, const SweepLaunch& L, int plane, int box_cols, int box_rows) {
   static PFN_cuTensorMapEncodeTiled_v12000 enc = nullptr;
   if (!enc) {
     void* fp = nullptr;
@@ -74,10 +74,13 @@ cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols,
   const cuuint64_t strides[1] = {static_cast<cuuint64_t>(L.pitch) * 4};
   const cuuint32_t box[2] = {static_cast<cuuint32_t>(box_cols), static_cast<cuuint32_t>(box_rows)};
   const cuuint32_t estr[2] = {1, 1};
-  CUresult r = enc(m, CU_TENSOR_MAP_DATA_TYPE_INT32, 2, L.out[0], dims, strides, box, estr,
+  CUresult r = enc(m, CU_TENSOR_MAP_DATA_TYPE_INT32, 2, L.out[plane], dims, strides, box, estr,
                    CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_NONE,
                    CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   return r == CUDA_SUCCESS ? cudaSuccess : cudaErrorInvalidValue;
+}
+cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols, int box_rows) {
+  return encode_plane_map_f(m, L, 0, box_cols, box_rows);
 }
 
 namespace {
@@ -174,12 +177,23 @@ bool want_nw7() {
   return e && e[0] == '7';
 }
 
+// SYNTHETIC at skew 1 runs the wf_syn.cu kernel unless WF_SYN_IMPL=4 (the generic sweep)
+bool want_syn7() {
+  const char* e = getenv("WF_SYN_IMPL");
+  return !(e && e[0] == '4');
+}
+
 const Variant* find(int fn, int dsize, int k, int warps, int skew) {
   size_t n;
   if (fn == WF_FN_SEQCMP && skew == 1 && want_nw7()) {
     const Variant* t7 = nw7_table(&n);
     for (size_t i = 0; i < n; ++i)
       if (t7[i].k == k && t7[i].warps == warps) return &t7[i];
+  }
+  if (fn == WF_FN_SYNTHETIC && skew == 1 && want_syn7()) {
+    const Variant* t7 = syn_table(&n);
+    for (size_t i = 0; i < n; ++i)
+      if (t7[i].dsize == dsize && t7[i].k == k && t7[i].warps == warps) return &t7[i];
   }
   const Variant* t = table(&n);
   for (size_t i = 0; i < n; ++i)

@@ -18,5 +18,7 @@ struct Variant {
 
 // SEQCMP v7 variants (wf_nw7.cu)
 const Variant* nw7_table(size_t* n);
+// SYNTHETIC v7 variants (wf_syn.cu)
+const Variant* syn_table(size_t* n);
 
 }  // namespace wfk

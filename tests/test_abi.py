@@ -106,8 +106,9 @@ def test_layout_slabs_partition_columns(dim, G):
 def test_nash_layout_one_column_per_warp():
     lay = query("nash", 4096, tsize=16, dsize=4)
     assert lay.nplanes == 4 and lay.nbound == 4 and lay.plane_is_float == [False] * 4
-    assert (lay.lane_cols, lay.warps, lay.skew) == (1, 8, 1)
-    assert lay.band_cols == 8 and lay.nbands == 512
+    # default band width follows the autotune winner for C3 (profiles/autotune_C3.json)
+    assert (lay.lane_cols, lay.warps, lay.skew) == (1, 2, 1)
+    assert lay.band_cols == 2 and lay.nbands == 2048
     lays = [query("nash", 4096, tsize=16, dsize=4, ngpus=2, rank=g) for g in range(2)]
     assert lays[0].col_end == lays[1].col_begin == 2048
 

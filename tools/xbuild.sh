@@ -7,9 +7,12 @@ NAME=$1; shift
 mkdir -p /tmp/wfx tools/abl_out
 N=/usr/local/cuda/bin/nvcc
 F="-gencode arch=compute_100a,code=sm_100a -O3 -lineinfo -std=c++17 -Xcompiler -fPIC --expt-relaxed-constexpr -Iinclude -Ipaper_conf_ppopp_mohantyc14_b200/csrc -DWF_MIN_VARIANTS"
-$N $F "$@" -c paper_conf_ppopp_mohantyc14_b200/csrc/wf_api.cpp -o /tmp/wfx/api_$NAME.o &
-$N $F "$@" -c paper_conf_ppopp_mohantyc14_b200/csrc/wf_nw7.cu -o /tmp/wfx/nw7_$NAME.o &
-$N $F "$@" -c paper_conf_ppopp_mohantyc14_b200/csrc/wf_sweep.cu -o /tmp/wfx/sweep_$NAME.o
+OBJS=""
+for s in paper_conf_ppopp_mohantyc14_b200/csrc/*.cu paper_conf_ppopp_mohantyc14_b200/csrc/*.cpp; do
+  o=/tmp/wfx/$(basename $s)_$NAME.o
+  $N $F "$@" -c $s -o $o &
+  OBJS="$OBJS $o"
+done
 wait
-$N -gencode arch=compute_100a,code=sm_100a -shared -cudart static -o tools/abl_out/libwf_$NAME.so /tmp/wfx/sweep_$NAME.o /tmp/wfx/nw7_$NAME.o /tmp/wfx/api_$NAME.o
+$N -gencode arch=compute_100a,code=sm_100a -shared -cudart static -o tools/abl_out/libwf_$NAME.so $OBJS
 echo tools/abl_out/libwf_$NAME.so
