@@ -284,9 +284,8 @@ def run_ours(args, cfg):
     w = Wavefront(cfg.fn, cfg.dim, rank=rank, device=local, ngpus=world, **fn_kwargs(cfg), **tun)
     lay = w.layout
     if world > 1:
-        handles = [None] * world
-        dist.all_gather_object(handles, w.ipc_handle())
-        w.connect(handles[rank - 1] if rank > 0 else None, handles[rank + 1] if rank < world - 1 else None)
+        from paper_conf_ppopp_mohantyc14_b200.dist import connect_slab
+        connect_slab(w, rank, world)   # all-gather of edge-ring IPC handles, wf_connect to g-1 / g+1
 
     inputs = host_inputs(cfg)
     if cfg.fn == "seqcmp":
@@ -336,9 +335,8 @@ def run_ours(args, cfg):
     step_ms_local = (sum(launch_ms) if flush else t_start.elapsed_time(t_end)) / args.steps
     avg_launch_ms = sum(launch_ms) / len(launch_ms)
     if world > 1:
-        tt = torch.tensor([step_ms_local], device=dev, dtype=torch.float64)
-        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
-        step_ms = float(tt.item())
+        from paper_conf_ppopp_mohantyc14_b200.dist import max_over_ranks
+        step_ms = max_over_ranks(step_ms_local, device=dev)
     else:
         step_ms = step_ms_local
     value = total_cells / (step_ms * 1e-3) / 1e9
@@ -361,9 +359,8 @@ def run_ours(args, cfg):
     w.sync()
     e2e_ms = e0.elapsed_time(e1) / e2e_steps
     if world > 1:
-        tt = torch.tensor([e2e_ms], device=dev, dtype=torch.float64)
-        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
-        e2e_ms = float(tt.item())
+        from paper_conf_ppopp_mohantyc14_b200.dist import max_over_ranks
+        e2e_ms = max_over_ranks(e2e_ms, device=dev)
     h2d = sum(p.numel() * p.element_size() for p in pinned)
     d2h = res_host.numel() * res_host.element_size()
 
