@@ -66,7 +66,9 @@ typedef enum {
    * P:732 ("Smith-Waterman"); Needleman-Wunsch global alignment with linear gap:
    *   H[i][0] = i*gap, H[0][j] = j*gap,
    *   H[i][j] = max(H[i-1][j-1] + (x_i == y_j ? match : mismatch), H[i-1][j] + gap, H[i][j-1] + gap)
-   * One int32 plane.  local = 1 (Smith-Waterman) is reserved: WF_EUNSUPPORTED. */
+   * One int32 plane.  local = 1: Smith-Waterman local alignment, H[i][0] = H[0][j] = 0,
+   *   H[i][j] = max(0, <the three terms above>); the run also reduces the first (row-major)
+   *   cell holding the maximum, read with wf_local_best. */
   WF_FN_SEQCMP = 2
 } wf_fn;
 
@@ -85,7 +87,7 @@ typedef struct {
   int32_t strip;        /* tunable: rows per inter-slab message (NCCL transport); 0 = default */
   int32_t ngpus;        /* slabs (column blocks), 1..8; see wf_dist */
   int32_t match, mismatch, gap;  /* SEQCMP scores, each in [-64, 64]; defaults used if all three 0 */
-  int32_t local;        /* SEQCMP: 0 = global (NW); 1 = local (SW): WF_EUNSUPPORTED in this ABI version */
+  int32_t local;        /* SEQCMP: 0 = global (Needleman-Wunsch), 1 = local (Smith-Waterman) */
   uint32_t transport;   /* wf_transport for ngpus > 1 */
   uint32_t max_ctas;    /* 0 = all resident CTAs; else an upper bound (tests of the band loop) */
   uint64_t watchdog_cycles; /* spin budget per dependency wait (SM clock cycles); 0 = default 2^32 */
@@ -183,6 +185,13 @@ wf_status wf_ipc_handle(struct wf_ctx* c, void* handle);
  * stored into its ring over NVLink.  WF_EINVAL if a required handle is missing, WF_ECOMM if
  * a handle cannot be opened. */
 wf_status wf_connect(struct wf_ctx* c, const void* prev_handle, const void* next_handle);
+
+/* SEQCMP local = 1 (Smith-Waterman): the best local
+ * alignment score of this slab's columns and its cell, the first in row-major order holding
+ * it -- 1-based row, 1-based GLOBAL column (a multi-slab caller takes the max over slabs,
+ * ties to the smallest (row, col)).  Blocks until the last run completed.  WF_ESTATE if the
+ * context is not local SEQCMP or has not run. */
+wf_status wf_local_best(struct wf_ctx* c, int32_t* score, int32_t* row, int32_t* col);
 
 /* Device time of the last completed run in milliseconds (CUDA events bracketing the
  * launch on the run's stream); WF_ESTATE if no run has completed. */

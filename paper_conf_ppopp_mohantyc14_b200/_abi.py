@@ -22,7 +22,8 @@ WF_TRANSPORT_P2P, WF_TRANSPORT_NCCL = 0, 1
 
 # every symbol include/wf.h declares (checked by tests/test_abi.py)
 EXPORTS = ("wf_query", "wf_create", "wf_run", "wf_sync", "wf_destroy", "wf_last_error", "wf_link_local",
-           "wf_ipc_handle", "wf_connect", "wf_last_run_ms", "wf_abi_version", "wf_build_info", "wf_debug_trace")
+           "wf_ipc_handle", "wf_connect", "wf_last_run_ms", "wf_abi_version", "wf_build_info", "wf_debug_trace",
+           "wf_local_best")
 
 
 class WfParams(ctypes.Structure):
@@ -84,6 +85,8 @@ def lib() -> ctypes.CDLL:
         L.wf_ipc_handle.argtypes = [P, P]
         L.wf_connect.argtypes = [P, P, P]
         L.wf_last_run_ms.argtypes = [P, ctypes.POINTER(ctypes.c_float)]
+        i32p = ctypes.POINTER(ctypes.c_int32)
+        L.wf_local_best.argtypes = [P, i32p, i32p, i32p]
         L.wf_debug_trace.argtypes = [P, P, ctypes.c_size_t, ctypes.POINTER(ctypes.c_int32)]
         L.wf_debug_trace.restype = ctypes.c_int
         L.wf_abi_version.argtypes = []
@@ -91,7 +94,7 @@ def lib() -> ctypes.CDLL:
         L.wf_build_info.argtypes = []
         L.wf_build_info.restype = ctypes.c_char_p
         for name in ("wf_query", "wf_create", "wf_run", "wf_sync", "wf_destroy", "wf_link_local",
-                     "wf_ipc_handle", "wf_connect", "wf_last_run_ms"):
+                     "wf_ipc_handle", "wf_connect", "wf_last_run_ms", "wf_local_best"):
             getattr(L, name).restype = ctypes.c_int
         _lib = L
     return _lib

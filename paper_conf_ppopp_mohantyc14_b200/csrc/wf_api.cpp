@@ -38,6 +38,8 @@ struct wf_ctx {
   void* next_ipc_base = nullptr;
   int* err = nullptr;                      // device error word
   unsigned long long* trace = nullptr;     // WF_TRACE=1 timeline buffer (diagnostics)
+  int2* lane_best = nullptr;               // local = 1: per-lane (best value, first row)
+  int32_t* best_out = nullptr;             // local = 1: the slab's best cell (value, row, col)
   uint32_t epoch = 0;
   cudaEvent_t ev0 = nullptr, ev1 = nullptr;
   bool ran = false;
@@ -115,7 +117,6 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
       if (p->tsize != 0) return fail(c, WF_EINVAL, "tsize=%d must be 0 for SEQCMP", p->tsize);
       if (p->dsize != 0) return fail(c, WF_EINVAL, "dsize=%d must be 0 for SEQCMP", p->dsize);
       if (p->local != 0 && p->local != 1) return fail(c, WF_EINVAL, "local=%d must be 0 or 1", p->local);
-      if (p->local == 1) return fail(c, WF_EUNSUPPORTED, "local=1 (Smith-Waterman) is not built in ABI v1");
       const bool def = p->match == 0 && p->mismatch == 0 && p->gap == 0;
       pl.match = def ? 1 : p->match;
       pl.mismatch = def ? -1 : p->mismatch;
@@ -148,7 +149,7 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   if (pl.k != 1 && pl.k != 2 && pl.k != 4 && pl.k != 8) return fail(c, WF_EINVAL, "lane_cols=%d not in {1,2,4,8}", pl.k);
   if (pl.warps < 1 || pl.warps > 8) return fail(c, WF_EINVAL, "warps=%d out of range 1..8", pl.warps);
   if (pl.skew < 1 || pl.skew > 4) return fail(c, WF_EINVAL, "skew=%d out of range 1..4", pl.skew);
-  if (!wfk::variant_exists(p->fn, p->dsize, pl.k, pl.warps, pl.skew))
+  if (!wfk::variant_exists(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew))
     return fail(c, WF_EUNSUPPORTED, "no kernel variant for fn=%d dsize=%d lane_cols=%d warps=%d skew=%d", p->fn,
                 p->dsize, pl.k, pl.warps, pl.skew);
   pl.band_w = p->fn == WF_FN_NASH ? pl.warps : pl.warps * 32 * pl.k;   // NASH: one column per warp
@@ -264,6 +265,7 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   wfk::SweepLaunch L{};
   L.fn = p->fn;
   L.dsize = p->dsize;
+  L.local = p->fn == WF_FN_SEQCMP ? p->local : 0;
   L.k = pl.k;
   L.warps = pl.warps;
   L.skew = pl.skew;
@@ -297,6 +299,11 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   }
   if (e == cudaSuccess) e = cudaMalloc(&c->err, sizeof(int));
   if (e == cudaSuccess) e = cudaMemset(c->err, 0, sizeof(int));
+  if (e == cudaSuccess && L.local) {   // Smith-Waterman best-cell reduction scratch
+    e = cudaMalloc(&c->lane_best, (size_t)pl.nbands * pl.warps * 32 * sizeof(int2));
+    if (e == cudaSuccess) e = cudaMalloc(&c->best_out, 4 * sizeof(int32_t));
+    if (e == cudaSuccess) e = cudaMemset(c->best_out, 0, 4 * sizeof(int32_t));
+  }
   if (e == cudaSuccess) e = cudaEventCreate(&c->ev0);
   if (e == cudaSuccess) e = cudaEventCreate(&c->ev1);
   if (e == cudaSuccess) e = cudaDeviceSynchronize();
@@ -319,6 +326,8 @@ wf_status wf_destroy(wf_ctx* c) {
   if (c->prev_ipc_base) cudaIpcCloseMemHandle(c->prev_ipc_base);
   if (c->base) cudaFree(c->base);
   if (c->err) cudaFree(c->err);
+  if (c->lane_best) cudaFree(c->lane_best);
+  if (c->best_out) cudaFree(c->best_out);
   if (c->trace) cudaFree(c->trace);
   if (c->ev0) cudaEventDestroy(c->ev0);
   if (c->ev1) cudaEventDestroy(c->ev1);
@@ -448,6 +457,9 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   L.cols = cols;
   L.tsize = p.tsize;
   L.dsize = p.dsize;
+  L.local = p.fn == WF_FN_SEQCMP ? p.local : 0;
+  L.lane_best = c->lane_best;
+  L.best_out = c->best_out;
   L.c0 = c->c0;
   L.c1 = c->c1;
   L.match = p.match;
@@ -490,6 +502,7 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   cudaStream_t s = static_cast<cudaStream_t>(cuda_stream);
   cudaError_t e = cudaEventRecord(c->ev0, s);
   if (e == cudaSuccess) e = wfk::launch(L, s);
+  if (e == cudaSuccess && L.local) e = wfk::launch_sw_best(L, s);   // part of the step: inside the timed events
   if (e == cudaSuccess) e = cudaEventRecord(c->ev1, s);
   if (prev >= 0 && prev != c->device) cudaSetDevice(prev);
   if (e != cudaSuccess) return cuda_fail(c, e, "wf_run launch");
@@ -518,6 +531,20 @@ wf_status wf_debug_trace(wf_ctx* c, void* host, size_t bytes, int32_t* slots_per
   const size_t need = (size_t)c->nbands * wfk::kTraceSlots * 8;
   cudaError_t e = cudaMemcpy(host, c->trace, bytes < need ? bytes : need, cudaMemcpyDeviceToHost);
   if (e != cudaSuccess) return cuda_fail(c, e, "wf_debug_trace");
+  return WF_OK;
+}
+
+wf_status wf_local_best(wf_ctx* c, int32_t* score, int32_t* row, int32_t* col) {
+  if (!c || !score || !row || !col) return fail(c, WF_EINVAL, "wf_local_best: NULL argument");
+  if (!(c->p.fn == WF_FN_SEQCMP && c->p.local == 1)) return fail(c, WF_ESTATE, "wf_local_best: context is not local SEQCMP");
+  if (!c->ran) return fail(c, WF_ESTATE, "wf_local_best: no run yet");
+  cudaError_t e = cudaEventSynchronize(c->ev1);
+  int32_t h[4] = {0, 0, 0, 0};
+  if (e == cudaSuccess) e = cudaMemcpy(h, c->best_out, sizeof h, cudaMemcpyDeviceToHost);
+  if (e != cudaSuccess) return cuda_fail(c, e, "wf_local_best");
+  *score = h[0];
+  *row = h[1];
+  *col = h[2];
   return WF_OK;
 }
 

@@ -42,6 +42,11 @@ struct SweepLaunch {
   // compute warp 0 lane 0 every rows/kTraceRows rows, plus feeder poll counters.
   unsigned long long* trace;
   unsigned long long watchdog;
+  // SEQCMP local = 1 (Smith-Waterman): per lane (best value, first row reaching it),
+  // [nbands][warps][32]; the slab's best cell (value, 1-based row, 1-based global column)
+  int32_t local;
+  int2* lane_best;
+  int32_t* best_out;
 };
 
 // LL slots per band ring and cell word: slot r holds row r (1..rows); padded to an even
@@ -56,7 +61,9 @@ int smem_bytes(const SweepLaunch& L);
 int occupancy(const SweepLaunch& L, int smem);
 // Launch (asynchronous).  Returns cudaSuccess or the launch error.
 cudaError_t launch(const SweepLaunch& L, cudaStream_t s);
-// Is (fn, dsize, k, warps, skew) compiled?
+// Finish the Smith-Waterman best-cell reduction of a run (after the sweep, same stream).
+cudaError_t launch_sw_best(const SweepLaunch& L, cudaStream_t s);
+// Is (fn, dsize, k, warps, skew) compiled?  (SEQCMP: dsize carries the local flag.)
 bool variant_exists(int fn, int dsize, int k, int warps, int skew);
 
 constexpr int kTraceSlots = 64;   // per band: [0..32] row stamps, [40] feeder polls, [41] empty polls,

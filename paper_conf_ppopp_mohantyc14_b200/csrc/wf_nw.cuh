@@ -104,7 +104,12 @@ __device__ __forceinline__ uint32_t lds_u8(const unsigned char* p) {
 // =====================================================================================
 // Compute warp: lane l owns K adjacent columns; at step t it is on row t - D*l + 1.
 // =====================================================================================
-template <int K, int WARPS, int D, int U, bool PRMT>
+// LOCAL = Smith-Waterman (R9): H = max(0, NW + s, N + g, W + g),
+// boundary 0.  The floor rides on the same VIADDMNMX (its .RELU form), so
+// max(t1_m, H_{m-1} + g) and the prefix form stay exact; the lane also tracks its best cell
+// value and the first row reaching it (the fused best-cell reduction, finished by
+// sw_best_kernel in wf_sw.cu).
+template <int K, int WARPS, int D, int U, bool PRMT, bool LOCAL = false>
 struct NwWarp {
   using S = NwSmem<K, WARPS, D, U>;
   static constexpr int R = S::R;
@@ -143,6 +148,12 @@ struct NwWarp {
   // published block (rows r31_0 .. r31_0+U-1) contiguous for the TMA box.
   int phase, ring_off;
   int seen_wprog, seen_rprog, seen_xfill;
+  int32_t best = 0;          // LOCAL: the lane's best cell value so far (cells are >= 0) ...
+  int32_t best_row = 0;      // ... and the first row reaching it (0: none above 0 yet)
+  __device__ __forceinline__ static int32_t t1f(int32_t N, int32_t g, int32_t d) {
+    if constexpr (LOCAL) return __viaddmax_s32_relu(N, g, d);   // max(N + g, d, 0)
+    else return __viaddmax_s32(N, g, d);
+  }
   Watchdog wd;
 
   __device__ __forceinline__ NwWarp(const SweepLaunch& L_, const CUtensorMap* tmap_, const S& sm_, int band_,
@@ -176,9 +187,9 @@ struct NwWarp {
       }
       qlo[m] = lo;
       qhi[m] = hi;
-      Np[m] = vc ? (jb + m + 1) * gap : 0;          // H[0][j] = j*g
+      Np[m] = (vc && !LOCAL) ? (jb + m + 1) * gap : 0;   // H[0][j] = j*g (NW), 0 (SW)
     }
-    prevW = jb < L.c1 ? jb * gap : 0;               // H[0][jb]
+    prevW = (jb < L.c1 && !LOCAL) ? jb * gap : 0;          // H[0][jb]
 #pragma unroll
     for (int d = 0; d < D; ++d) {
       q[d] = 0;
@@ -220,7 +231,7 @@ struct NwWarp {
         int32_t s;
         if constexpr (PRMT) s = prmt_s8(qlo[m], qhi[m], sel);
         else s = (xc == ycode[m]) ? mmatch : mmis;
-        const int32_t t1 = __viaddmax_s32(Np[m], gap, NW + s);
+        const int32_t t1 = t1f(Np[m], gap, NW + s);
         P = (m == 0) ? t1 : __viaddmax_s32(P, gap, t1);
         H[m] = __viaddmax_s32(Win, gk[m], P);
       }
@@ -232,7 +243,7 @@ struct NwWarp {
         int32_t s;
         if constexpr (PRMT) s = prmt_s8(qlo[m], qhi[m], sel);
         else s = (xc == ycode[m]) ? mmatch : mmis;
-        const int32_t t1 = __viaddmax_s32(Np[m], gap, NW + s);
+        const int32_t t1 = t1f(Np[m], gap, NW + s);
         H[m] = __viaddmax_s32(W, gap, t1);
       }
     }
@@ -347,7 +358,7 @@ struct NwWarp {
       int32_t s;
       if constexpr (PRMT) s = prmt_s8(qlo[m], qhi[m], sel);
       else s = (xc == ycode[m]) ? mmatch : mmis;
-      const int32_t t1 = __viaddmax_s32(Np[m], gap, NW + s);
+      const int32_t t1 = t1f(Np[m], gap, NW + s);
       P = (m == 0) ? t1 : __viaddmax_s32(P, gap, t1);
       H[m] = __viaddmax_s32(Win, gk[m], P);
     }
@@ -369,6 +380,14 @@ struct NwWarp {
       const uint32_t Xin = (lane == 0) ? x0 : xq[D - 1];
       int32_t H[K];
       cells(Win, Xin, H);
+      if constexpr (LOCAL) {   // best cell: strict > keeps the first row reaching the value
+        int32_t rm = H[0];
+#pragma unroll
+        for (int m = 1; m < K; ++m) rm = max(rm, H[m]);
+        const bool up = rm > best && (!EDGE || (row >= 1 && row <= rows));
+        best = up ? rm : best;
+        best_row = up ? row : best_row;
+      }
       if constexpr (EDGE) {   // ramp-up / drain: predicated selects, no divergent branch
         const bool active = row >= 1 && row <= rows;
         prevW = active ? Win : prevW;
@@ -487,6 +506,7 @@ struct NwWarp {
       L.trace[size_t(band) * kTraceSlots + kTraceRows] = globaltimer();
       L.trace[size_t(band) * kTraceSlots + 43] = clock64();
     }
+    if constexpr (LOCAL) L.lane_best[(size_t(band) * WARPS + warp) * 32 + lane] = make_int2(best, best_row);
     return true;
   }
 };
@@ -494,7 +514,7 @@ struct NwWarp {
 // =====================================================================================
 // I/O warp: x staging, west feed of warp 0, east forwarding of warp WARPS-1.
 // =====================================================================================
-template <int K, int WARPS, int D, int U>
+template <int K, int WARPS, int D, int U, bool LOCAL = false>
 __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K, WARPS, D, U>& sm, int band,
                                            int lane) {
   using S = NwSmem<K, WARPS, D, U>;
@@ -529,7 +549,7 @@ __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K,
           v[h] = 0;
           if (r <= rows) {
             if (boundary) {
-              v[h] = r * L.gap;                                   // H[r][0] = r*g
+              v[h] = LOCAL ? 0 : r * L.gap;                       // H[r][0] = r*g (NW), 0 (SW)
             } else {
               const unsigned long long wv = ld_relaxed_sys(src + r);
               v[h] = static_cast<int32_t>(static_cast<uint32_t>(wv));
@@ -631,7 +651,7 @@ __device__ __forceinline__ bool nw_x_warp(const SweepLaunch& L, const NwSmem<K, 
   return true;
 }
 
-template <int K, int WARPS, int D, int U, bool PRMT>
+template <int K, int WARPS, int D, int U, bool PRMT, bool LOCAL = false>
 __global__ void __launch_bounds__((WARPS + 2) * 32)
     nw_kernel(const SweepLaunch L, const PolSeq pol, const __grid_constant__ CUtensorMap tmap) {
   using S = NwSmem<K, WARPS, D, U>;
@@ -645,9 +665,9 @@ __global__ void __launch_bounds__((WARPS + 2) * 32)
     if (warp == WARPS + 1) {
       nw_x_warp<K, WARPS, D, U>(L, sm, lane);
     } else if (warp == WARPS) {
-      nw_io_warp<K, WARPS, D, U>(L, sm, band, lane);
+      nw_io_warp<K, WARPS, D, U, LOCAL>(L, sm, band, lane);
     } else {
-      NwWarp<K, WARPS, D, U, PRMT> w(L, &tmap, sm, band, warp, lane);
+      NwWarp<K, WARPS, D, U, PRMT, LOCAL> w(L, &tmap, sm, band, warp, lane);
       w.run();
     }
     __syncthreads();

@@ -185,6 +185,12 @@ bool want_syn7() {
 
 const Variant* find(int fn, int dsize, int k, int warps, int skew) {
   size_t n;
+  if (fn == WF_FN_SEQCMP && dsize == 1) {   // local alignment (Smith-Waterman)
+    const Variant* ts = sw_table(&n);
+    for (size_t i = 0; i < n; ++i)
+      if (ts[i].k == k && ts[i].warps == warps && ts[i].skew == skew) return &ts[i];
+    return nullptr;
+  }
   if (fn == WF_FN_SEQCMP && skew == 1 && want_nw7()) {
     const Variant* t7 = nw7_table(&n);
     for (size_t i = 0; i < n; ++i)
@@ -205,19 +211,19 @@ const Variant* find(int fn, int dsize, int k, int warps, int skew) {
 
 bool variant_exists(int fn, int dsize, int k, int warps, int skew) {
   // compiled AND within the 227 KB per-CTA shared-memory limit of sm_100
-  const Variant* v = find(fn, fn == WF_FN_SYNTHETIC ? dsize : 0, k, warps, skew);
+  const Variant* v = find(fn, (fn == WF_FN_SYNTHETIC || fn == WF_FN_SEQCMP) ? dsize : 0, k, warps, skew);
   return v != nullptr && v->smem <= 232448;
 }
 
 int smem_bytes(const SweepLaunch& L) {
-  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : 0, L.k, L.warps, L.skew);
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew);
   if (!v) return -1;
   if (L.fn == WF_FN_NASH) return (int)(v->smem + size_t(L.warps) * ((size_t(2) * L.tsize * L.tsize + 2 * L.tsize + 15) & ~size_t(15)));
   return (int)v->smem;
 }
 
 int occupancy(const SweepLaunch& L, int smem) {
-  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : 0, L.k, L.warps, L.skew);
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew);
   if (!v) return 0;
   if (cudaFuncSetAttribute(v->kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem) != cudaSuccess) {
     cudaGetLastError();
@@ -232,7 +238,7 @@ int occupancy(const SweepLaunch& L, int smem) {
 }
 
 cudaError_t launch(const SweepLaunch& L, cudaStream_t s) {
-  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : 0, L.k, L.warps, L.skew);
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew);
   if (!v) return cudaErrorInvalidDeviceFunction;
   return v->launch(L, s, (size_t)smem_bytes(L));
 }

@@ -18,6 +18,8 @@ struct Variant {
 
 // SEQCMP v7 variants (wf_nw7.cu)
 const Variant* nw7_table(size_t* n);
+// SEQCMP local (Smith-Waterman) variants (wf_sw.cu); looked up with dsize = 1
+const Variant* sw_table(size_t* n);
 // SYNTHETIC v7 variants (wf_syn.cu)
 const Variant* syn_table(size_t* n);
 

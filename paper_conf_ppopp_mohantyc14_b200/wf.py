@@ -142,6 +142,13 @@ class Wavefront:
     def sync(self) -> None:
         check(_abi.lib().wf_sync(self._ctx), self._ctx)
 
+    def local_best(self) -> tuple[int, int, int]:
+        """Smith-Waterman (local=1): (best score, 1-based row, 1-based global column) of the
+        first cell in row-major order holding it, from the last run (wf_local_best)."""
+        v, r, c = ctypes.c_int32(), ctypes.c_int32(), ctypes.c_int32()
+        check(_abi.lib().wf_local_best(self._ctx, ctypes.byref(v), ctypes.byref(r), ctypes.byref(c)), self._ctx)
+        return int(v.value), int(r.value), int(c.value)
+
     def last_run_ms(self) -> float:
         ms = ctypes.c_float()
         check(_abi.lib().wf_last_run_ms(self._ctx, ctypes.byref(ms)), self._ctx)

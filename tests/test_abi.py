@@ -76,9 +76,11 @@ def test_reserved_fields_must_be_zero():
     assert st == _abi.WF_EINVAL and b"reserved" in _abi.lib().wf_last_error(None)
 
 
-def test_local_alignment_is_reported_unsupported():
-    e = _err("seqcmp", 64, local=1)
-    assert e.status == _abi.WF_EUNSUPPORTED
+def test_local_alignment_layout_and_bad_flag():
+    # Smith-Waterman (local = 1) is built: same single int32 plane as global alignment
+    lay = query("seqcmp", 64, local=1)
+    assert lay.nplanes == 1 and lay.plane_is_float == [False]
+    assert _err("seqcmp", 64, local=2).status == _abi.WF_EINVAL
 
 
 def test_layout_single_slab():

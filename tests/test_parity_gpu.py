@@ -74,6 +74,71 @@ def test_seqcmp_v7_local_slabs(monkeypatch, G):
     assert np.array_equal(H, g)
 
 
+def _sw_expect(H):
+    """Best local score and its first cell in row-major order (1-based), by definition."""
+    flat = int(np.argmax(H))
+    r, c = divmod(flat, H.shape[1])
+    return int(H.flat[flat]), r + 1, c + 1
+
+
+def _sw_run(dim, cols=0, kind="random", scoring=(2, -1, -1), seed=(1, 2), **kw):
+    n = cols or dim
+    x, y = workloads.seqcmp_inputs(dim, n, kind=kind, seed_x=seed[0], seed_y=seed[1])
+    M, X, G = scoring
+    H = oracle.seqcmp(x, y, M, X, G, local=True)
+    dev = torch.device("cuda", torch.cuda.current_device())
+    with Wavefront("seqcmp", dim, cols=cols, match=M, mismatch=X, gap=G, local=1, **kw) as w:
+        row_in, col_in, top, left = dev_inputs("seqcmp", (x, y), dev)
+        (g,) = w.run(row_in, col_in, top, left)
+        w.sync()
+        best = w.local_best()
+        g = g.cpu().numpy()
+    return H, g, best
+
+
+@pytest.mark.parametrize("dim", [1, 2, 7, 33, 64, 97, 300, 777, 1100])
+@pytest.mark.parametrize("scoring", [(2, -1, -1), (1, -1, -1), (3, -2, -2), (-1, -1, -1)])
+def test_smith_waterman_grid_and_best_cell(dim, scoring):
+    H, g, best = _sw_run(dim, scoring=scoring, seed=(dim + 11, dim + 12), alphabet=4)
+    assert np.array_equal(H, g)
+    assert best == _sw_expect(H)
+
+
+@pytest.mark.parametrize("k,w,d", [(4, 2, 1), (4, 1, 1), (2, 2, 1), (2, 4, 1), (8, 1, 1), (4, 1, 2), (2, 2, 2), (1, 2, 1)])
+@pytest.mark.parametrize("alphabet", [0, 4])
+def test_smith_waterman_variants(k, w, d, alphabet):
+    for dim, cols in ((1000, 0), (513, 1200), (1300, 257)):
+        H, g, best = _sw_run(dim, cols=cols, lane_cols=k, warps=w, skew=d, alphabet=alphabet, seed=(dim, cols + 3))
+        assert np.array_equal(H, g)
+        assert best == _sw_expect(H)
+
+
+def test_smith_waterman_related_sequences_best_cell():
+    # a 10%-mutated copy: a long diagonal of matches, best cell far from the start
+    H, g, best = _sw_run(2000, kind="mutated", scoring=(1, -1, -1), alphabet=4)
+    assert np.array_equal(H, g)
+    assert best == _sw_expect(H) and best[0] > 1000
+
+
+def test_smith_waterman_c4_size_best_cell():
+    """C4 shape (dim 32768, 1 Gi cells) in the bench launch configuration: the best cell
+    against the oracle's rows up to it (an exact row prefix), and the grid's last row."""
+    dim = 32768
+    x, y = workloads.seqcmp_inputs(dim, dim, kind="mutated")
+    dev = torch.device("cuda", torch.cuda.current_device())
+    with Wavefront("seqcmp", dim, match=1, mismatch=-1, gap=-1, local=1, alphabet=4) as w:
+        row_in, col_in, top, left = dev_inputs("seqcmp", (x, y), dev)
+        (g,) = w.run(row_in, col_in, top, left)
+        w.sync()
+        v, r, c = w.local_best()
+        last = g[-1].cpu().numpy()
+        assert int(g[r - 1, c - 1].item()) == v
+        del g
+    want = oracle.seqcmp(x, y, 1, -1, -1, local=True)
+    assert np.array_equal(last, want[-1])
+    assert (v, r, c) == _sw_expect(want)
+
+
 @pytest.mark.parametrize("alphabet", [4, 8])
 @pytest.mark.parametrize("scoring", [(1, -1, -1), (2, -3, -1), (-3, 2, -1), (64, -64, -64), (-64, 64, 64)])
 def test_seqcmp_byte_permute_scores(alphabet, scoring):
