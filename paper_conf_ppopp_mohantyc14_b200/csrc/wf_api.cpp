@@ -88,8 +88,10 @@ void defaults(const wf_params& p, int* k, int* w, int* d) {
     // synthetic (wf_syn.cu): one column per lane keeps the tsize-deep FMA chain per step
     // short; one compute warp per CTA (32-column bands, several CTAs per SM share its
     // SMSPs) measured fastest on C5a/C5b (tools/autotune.py, profiles/autotune_*.json)
+    // -- except many items with a deep chain (dsize >= 5, tsize >= 1000: C5d), where the
+    // generic sweep with 4 warps won (154.6 vs 196.7 ms, profiles/autotune_C5d.json)
     *k = p.lane_cols ? p.lane_cols : 1;
-    *w = p.warps ? p.warps : 1;
+    *w = p.warps ? p.warps : ((p.dsize >= 5 && p.tsize >= 1000) ? 4 : 1);
     *d = p.skew ? p.skew : 1;
   }
 }

@@ -45,6 +45,7 @@ struct SweepLaunch {
   // SEQCMP local = 1 (Smith-Waterman): per lane (best value, first row reaching it),
   // [nbands][warps][32]; the slab's best cell (value, 1-based row, 1-based global column)
   int32_t local;
+  int32_t cluster;     // SEQCMP v4: launched as clusters of 8 CTAs, band-to-band hand-off via DSMEM
   int2* lane_best;
   int32_t* best_out;
 };

@@ -95,6 +95,37 @@ __device__ __forceinline__ int32_t lds_vol_s32(const void* p) {
   asm volatile("ld.volatile.shared.s32 %0, [%1];" : "=r"(v) : "r"(static_cast<uint32_t>(__cvta_generic_to_shared(p))));
   return v;
 }
+// Distributed shared memory (thread-block clusters): the address of the same shared
+// variable in CTA `rank` of this cluster, and relaxed / release accesses to it.
+__device__ __forceinline__ uint32_t dsmem_addr(const void* local, uint32_t rank) {
+  uint32_t r;
+  asm volatile("mapa.shared::cluster.u32 %0, %1, %2;"
+               : "=r"(r)
+               : "r"(static_cast<uint32_t>(__cvta_generic_to_shared(local))), "r"(rank));
+  return r;
+}
+__device__ __forceinline__ void st_cluster_u32(uint32_t a, uint32_t v) {
+  asm volatile("st.relaxed.cluster.shared::cluster.u32 [%0], %1;" ::"r"(a), "r"(v) : "memory");
+}
+__device__ __forceinline__ void st_release_cluster_u32(uint32_t a, uint32_t v) {
+  asm volatile("st.release.cluster.shared::cluster.u32 [%0], %1;" ::"r"(a), "r"(v) : "memory");
+}
+__device__ __forceinline__ uint32_t ld_cluster_u32(uint32_t a) {
+  uint32_t v;
+  asm volatile("ld.relaxed.cluster.shared::cluster.u32 %0, [%1];" : "=r"(v) : "r"(a) : "memory");
+  return v;
+}
+__device__ __forceinline__ void fence_acq_rel_cluster() { asm volatile("fence.acq_rel.cluster;" ::: "memory"); }
+__device__ __forceinline__ void cluster_sync_all() {
+  asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
+}
+__device__ __forceinline__ uint32_t cluster_ctarank() {
+  uint32_t r;
+  asm volatile("mov.u32 %0, %%cluster_ctarank;" : "=r"(r));
+  return r;
+}
+constexpr int kClusterSize = 8;   // largest (portable) cluster size; L.cluster holds the launched size
+
 __device__ __forceinline__ uint32_t lds_u8(const unsigned char* p) {
   uint32_t v;
   asm volatile("ld.volatile.shared.u8 %0, [%1];" : "=r"(v) : "r"(static_cast<uint32_t>(__cvta_generic_to_shared(p))));
@@ -109,7 +140,7 @@ __device__ __forceinline__ uint32_t lds_u8(const unsigned char* p) {
 // max(t1_m, H_{m-1} + g) and the prefix form stay exact; the lane also tracks its best cell
 // value and the first row reaching it (the fused best-cell reduction, finished by
 // sw_best_kernel in wf_sw.cu).
-template <int K, int WARPS, int D, int U, bool PRMT, bool LOCAL = false>
+template <int K, int WARPS, int D, int U, bool PRMT, bool LOCAL = false, bool CL = false>
 struct NwWarp {
   using S = NwSmem<K, WARPS, D, U>;
   static constexpr int R = S::R;
@@ -281,9 +312,22 @@ struct NwWarp {
     if (seen >= need) return true;
     wd.start();
     for (;;) {
-      seen = lds_vol_i(ctr);
+      if constexpr (CL) {   // acquire at cluster scope: the feed counter may be released by the previous CTA
+        uint32_t v;
+        asm volatile("ld.acquire.cluster.shared::cta.u32 %0, [%1];"
+                     : "=r"(v)
+                     : "r"(static_cast<uint32_t>(__cvta_generic_to_shared(ctr)))
+                     : "memory");
+        seen = static_cast<int>(v);
+        if (seen >= need) return true;
+      } else {
+        seen = lds_vol_i(ctr);
+      }
       if (seen >= need) {
-        __threadfence_block();   // order the data reads after the observed counter
+        // order the data reads after the observed counter (cluster scope: the feed ring may be
+        // written by the previous band's CTA through DSMEM)
+        if constexpr (CL) fence_acq_rel_cluster();
+        else __threadfence_block();
         return true;
       }
       if (wd.expired(L)) return false;
@@ -514,7 +558,7 @@ struct NwWarp {
 // =====================================================================================
 // I/O warp: x staging, west feed of warp 0, east forwarding of warp WARPS-1.
 // =====================================================================================
-template <int K, int WARPS, int D, int U, bool LOCAL = false>
+template <int K, int WARPS, int D, int U, bool LOCAL = false, bool CL = false>
 __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K, WARPS, D, U>& sm, int band,
                                            int lane) {
   using S = NwSmem<K, WARPS, D, U>;
@@ -527,9 +571,21 @@ __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K,
   const unsigned char* east_col = sm.stage + size_t(WARPS - 1) * S::R * S::ROWB + (32 * K - 1) * 4;
   const int last_off = NwWarp<K, WARPS, D, U, true>::ring_offset(
       WF_NW_GLOBAL_PHASE ? (L.c0 / L.band_w + band) * WARPS + WARPS - 1 : WARPS - 1);
-  int feed = 1;                 // next row to feed
+  // Cluster mode: the previous band of this round runs in the CTA of cluster rank - 1 and
+  // writes this CTA's feed ring itself (DSMEM); this band's east column goes to rank + 1.
+  const uint32_t crank = CL ? cluster_ctarank() : 0u;
+  const bool from_cluster = CL && crank > 0 && band > 0;
+  const bool to_cluster = CL && crank + 1 < static_cast<uint32_t>(L.cluster) && band + 1 < L.nbands &&
+                          blockIdx.x + 1 < gridDim.x;
+  uint32_t r_feed = 0, r_wprog = 0, r_rprog = 0;
+  if (to_cluster) {
+    r_feed = dsmem_addr(sm.feed, crank + 1);
+    r_wprog = dsmem_addr(sm.wprog + WARPS, crank + 1);
+    r_rprog = dsmem_addr(sm.rprog + WARPS, crank + 1);
+  }
+  int feed = from_cluster ? rows + 1 : 1;   // next row to feed (the producer feeds a cluster band)
   int fwd = 1;                  // next row to forward from the last warp's staging ring
-  int seen_feed_rd = 0, seen_last_wr = 0;
+  int seen_feed_rd = 0, seen_last_wr = 0, seen_remote_rd = 0;
   bool acked = !wait_ack;
   Watchdog wd;
   wd.start();
@@ -590,15 +646,22 @@ __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K,
           seen_last_wr = lds_vol_i(sm.wprog + WARPS - 1);
           if (seen_last_wr >= fwd) __threadfence_block();
         }
-        const int avail = min(seen_last_wr, rows) - fwd + 1;
+        int avail = min(seen_last_wr, rows) - fwd + 1;
+        if (to_cluster && avail > 0) {   // the consumer's feed-ring slots must be free
+          const int need = fwd + min(avail, 32) - 1 - kFeed;
+          if (seen_remote_rd < need) seen_remote_rd = static_cast<int>(ld_cluster_u32(r_rprog));
+          if (seen_remote_rd < need) avail = 0;
+        }
         if (avail > 0) {
           const int n = min(avail, 32);
           const int r = fwd + lane;
           if (lane < n) {
             const int32_t v = lds_vol_s32(east_col + ((r + last_off) & (S::R - 1)) * S::ROWB);
-            if (dst) st_relaxed_sys(dst + r, ll_pack(static_cast<uint32_t>(v), L.epoch));
+            if (to_cluster) st_cluster_u32(r_feed + 4u * (r & (kFeed - 1)), static_cast<uint32_t>(v));
+            else if (dst) st_relaxed_sys(dst + r, ll_pack(static_cast<uint32_t>(v), L.epoch));
           }
-          __syncwarp();
+          __syncwarp();   // orders every lane's DSMEM store before lane 0's release of the counter
+          if (to_cluster && lane == 0) st_release_cluster_u32(r_wprog, static_cast<uint32_t>(fwd + n - 1));
           fwd += n;
           if (lane == 0) sts_vol_i(sm.rprog + WARPS - 1, fwd - 1);
           if (L.trace && lane == 0 && fwd - n <= 32 && fwd > 32)     // first 32 rows forwarded
@@ -651,7 +714,7 @@ __device__ __forceinline__ bool nw_x_warp(const SweepLaunch& L, const NwSmem<K, 
   return true;
 }
 
-template <int K, int WARPS, int D, int U, bool PRMT, bool LOCAL = false>
+template <int K, int WARPS, int D, int U, bool PRMT, bool LOCAL = false, bool CL = false>
 __global__ void __launch_bounds__((WARPS + 2) * 32)
     nw_kernel(const SweepLaunch L, const PolSeq pol, const __grid_constant__ CUtensorMap tmap) {
   using S = NwSmem<K, WARPS, D, U>;
@@ -659,6 +722,31 @@ __global__ void __launch_bounds__((WARPS + 2) * 32)
   const S sm(nw_smem_raw);
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   (void)pol;
+  if constexpr (CL) {
+    // every CTA of a cluster runs the same rounds (cluster barriers must match)
+    const int rounds = (L.nbands + gridDim.x - 1) / gridDim.x;
+    bool failed = false;
+    for (int round = 0; round < rounds; ++round) {
+      const int band = blockIdx.x + round * gridDim.x;
+      if (threadIdx.x < 64) reinterpret_cast<int*>(sm.wprog)[threadIdx.x] = 0;
+      __syncthreads();
+      cluster_sync_all();   // the neighbour's rings are initialised before any DSMEM store
+      if (band < L.nbands && !failed) {
+        if (warp == WARPS + 1) {
+          nw_x_warp<K, WARPS, D, U>(L, sm, lane);
+        } else if (warp == WARPS) {
+          nw_io_warp<K, WARPS, D, U, LOCAL, true>(L, sm, band, lane);
+        } else {
+          NwWarp<K, WARPS, D, U, PRMT, LOCAL, true> w(L, &tmap, sm, band, warp, lane);
+          w.run();
+        }
+      }
+      __syncthreads();
+      failed = failed || run_failed(L);
+      cluster_sync_all();   // no CTA leaves (or re-initialises) while a neighbour may still store into it
+    }
+    return;
+  } else {
   for (int band = blockIdx.x; band < L.nbands; band += gridDim.x) {
     if (threadIdx.x < 64) reinterpret_cast<int*>(sm.wprog)[threadIdx.x] = 0;   // wprog, rprog, xneed, xfill
     __syncthreads();
@@ -672,6 +760,7 @@ __global__ void __launch_bounds__((WARPS + 2) * 32)
     }
     __syncthreads();
     if (run_failed(L)) return;
+  }
   }
 }
 

@@ -85,6 +85,58 @@ cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols,
 
 namespace {
 
+}  // namespace
+
+// Launch an NW-family kernel.  With a cluster kernel `kcl` and WF_NW_CLUSTER=<size> (2, 4 or 8)
+// the grid is launched as clusters of that many CTAs (band-to-band hand-off through
+// distributed shared memory, wf_nw.cuh) when a whole number of co-resident clusters covers
+// the grid; otherwise as a plain persistent grid (the default: measured faster).
+cudaError_t launch_nw_kernel(void (*kfn)(const SweepLaunch, const PolSeq, const CUtensorMap),
+                             void (*kcl)(const SweepLaunch, const PolSeq, const CUtensorMap), const SweepLaunch& L,
+                             const PolSeq& pol, const CUtensorMap& tmap, int threads, size_t smem, cudaStream_t s) {
+  const char* env = getenv("WF_NW_CLUSTER");
+  const int cs = env ? atoi(env) : 0;
+  if (kcl && (cs == 2 || cs == 4 || cs == 8) && L.nbands >= 2 * cs && L.grid >= 2 * cs) {
+    cudaError_t e = cudaFuncSetAttribute(kcl, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    if (e != cudaSuccess) return e;
+    cudaLaunchConfig_t cfg = {};
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeClusterDimension;
+    at[0].val.clusterDim.x = cs;
+    at[0].val.clusterDim.y = 1;
+    at[0].val.clusterDim.z = 1;
+    cfg.blockDim = dim3(threads);
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = s;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    int g = (L.grid / cs) * cs;
+    cfg.gridDim = dim3(g);
+    int ncl = 0;
+    if (cudaOccupancyMaxActiveClusters(&ncl, reinterpret_cast<const void*>(kcl), &cfg) != cudaSuccess) {
+      cudaGetLastError();
+      ncl = 0;
+    }
+    if (getenv("WF_NW_CLUSTER_DEBUG")) fprintf(stderr, "wf: cluster %d launch grid %d, max active clusters %d\n", cs, g, ncl);
+    g = g < ncl * cs ? g : ncl * cs;
+    if (g >= 2 * cs) {
+      SweepLaunch Lc = L;
+      Lc.grid = g;
+      Lc.cluster = cs;
+      cfg.gridDim = dim3(g);
+      e = cudaLaunchKernelEx(&cfg, kcl, Lc, pol, tmap);
+      if (e == cudaSuccess) return cudaGetLastError();
+      cudaGetLastError();
+    }
+  }
+  SweepLaunch Lp = L;
+  Lp.cluster = 0;
+  kfn<<<L.grid, threads, smem, s>>>(Lp, pol, tmap);
+  return cudaGetLastError();
+}
+
+namespace {
+
 template <int K, int W, int D, int U>
 cudaError_t launch_nw(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   PolSeq pol{};
@@ -102,8 +154,11 @@ cudaError_t launch_nw(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   auto kfn = (L.alphabet >= 1 && L.alphabet <= 8) ? nw_kernel<K, W, D, U, true> : nw_kernel<K, W, D, U, false>;
   e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
-  kfn<<<L.grid, (W + 2) * 32, smem, s>>>(L, pol, tmap);   // + I/O warp + x-staging warp
-  return cudaGetLastError();
+  decltype(kfn) kcl = nullptr;
+  if constexpr (K == 4 && W == 2 && D == 1)   // the default C4 variant also exists as a cluster kernel
+    kcl = (L.alphabet >= 1 && L.alphabet <= 8) ? nw_kernel<K, W, D, U, true, false, true>
+                                               : nw_kernel<K, W, D, U, false, false, true>;
+  return launch_nw_kernel(kfn, kcl, L, pol, tmap, (W + 2) * 32, smem, s);   // + I/O warp + x-staging warp
 }
 
 template <int K, int W, int D>
@@ -198,8 +253,8 @@ const Variant* find(int fn, int dsize, int k, int warps, int skew) {
   }
   if (fn == WF_FN_SYNTHETIC && skew == 1 && want_syn7()) {
     const Variant* t7 = syn_table(&n);
-    for (size_t i = 0; i < n; ++i)
-      if (t7[i].dsize == dsize && t7[i].k == k && t7[i].warps == warps) return &t7[i];
+    for (size_t i = 0; i < n; ++i)   // a wf_syn variant whose staging rings do not fit falls back to the generic sweep
+      if (t7[i].dsize == dsize && t7[i].k == k && t7[i].warps == warps && t7[i].smem <= 232448) return &t7[i];
   }
   const Variant* t = table(&n);
   for (size_t i = 0; i < n; ++i)
