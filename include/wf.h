@@ -94,7 +94,10 @@ typedef struct {
   int32_t alphabet;     /* SEQCMP: 0 = residue codes may be any byte value; 1..8 = every code in
                            row_in/col_in is < alphabet (e.g. 4 for DNA) -- enables the byte-permute
                            score lookup; codes outside the promise give unspecified scores */
-  int32_t reserved[5];  /* must be zero */
+  int32_t kernel;       /* kernel generation: 0 = the library's default for the function (tuned, DESIGN.md
+                           §7); 4 = first generation (SEQCMP block hand-off v4, SYNTHETIC generic sweep);
+                           7 = second generation (SEQCMP per-row hand-off v7, SYNTHETIC wf_syn) */
+  int32_t reserved[4];  /* must be zero */
 } wf_params;
 
 /* Distribution: which slab this context computes.

@@ -28,6 +28,7 @@ struct wf_ctx {
   int k = 4, warps = 2, skew = 2, band_w = 256, nbands = 1;
   int grid = 1;
   int smem = 0;
+  int impl = 0;
   void* base = nullptr;                    // one allocation: [control block | edge rings] (IPC-exportable)
   unsigned* ack = nullptr;                 // control word written by the successor slab
   unsigned long long* edge = nullptr;      // nbands * rows * nf LL words (library-owned)
@@ -69,11 +70,13 @@ wf_status cuda_fail(wf_ctx* c, cudaError_t e, const char* what) {
 
 struct Plan {
   int nf, nbound, k, warps, skew, band_w, c0, c1, nbands;
+  int impl;   // kernel generation actually used (wf_params.kernel, or the default's)
   int match, mismatch, gap;
 };
 
 // Defaults until the autotune table says otherwise (tools/autotune.py).
-void defaults(const wf_params& p, int* k, int* w, int* d) {
+void defaults(const wf_params& p, int* k, int* w, int* d, int* impl) {
+  *impl = p.kernel;
   if (p.fn == WF_FN_SEQCMP) {
     *k = p.lane_cols ? p.lane_cols : 4;
     *w = p.warps ? p.warps : 2;
@@ -85,14 +88,16 @@ void defaults(const wf_params& p, int* k, int* w, int* d) {
     *w = p.warps ? p.warps : 2;
     *d = p.skew ? p.skew : 1;
   } else {
-    // synthetic (wf_syn.cu): one column per lane keeps the tsize-deep FMA chain per step
-    // short; one compute warp per CTA (32-column bands, several CTAs per SM share its
-    // SMSPs) measured fastest on C5a/C5b (tools/autotune.py, profiles/autotune_*.json)
-    // -- except many items with a deep chain (dsize >= 5, tsize >= 1000: C5d), where the
-    // generic sweep with 4 warps won (154.6 vs 196.7 ms, profiles/autotune_C5d.json)
+    // synthetic: one column per lane keeps the tsize-deep FMA chain per step short.  From the
+    // B200 sweep (profiles/tuner_sweep.json, 27 instances x all variants): one compute warp per
+    // CTA with wf_syn for light cells; when a cell carries much FP work (dsize >= 3 with
+    // tsize >= 1000, or dsize >= 5 with tsize >= 100) the generic sweep with 2 (dsize 3) or
+    // 4 (dsize >= 5) warps per CTA wins (e.g. C5d 154 vs 197 ms).
+    const bool heavy = (p.dsize >= 3 && p.tsize >= 1000) || (p.dsize >= 5 && p.tsize >= 100);
     *k = p.lane_cols ? p.lane_cols : 1;
-    *w = p.warps ? p.warps : ((p.dsize >= 5 && p.tsize >= 1000) ? 4 : 1);
+    *w = p.warps ? p.warps : (heavy ? (p.dsize >= 5 ? 4 : 2) : 1);
     *d = p.skew ? p.skew : 1;
+    if (!p.kernel && heavy && !p.warps && !p.lane_cols) *impl = 4;
   }
 }
 
@@ -102,7 +107,9 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   const int cols = p->cols ? p->cols : p->dim;
   if (rows < 1 || rows > 65535) return fail(c, WF_EINVAL, "dim=%d out of range 1..65535", rows);
   if (cols < 1 || cols > 65535) return fail(c, WF_EINVAL, "cols=%d out of range 1..65535", cols);
-  for (int i = 0; i < 5; ++i)
+  if (p->kernel != 0 && p->kernel != 4 && p->kernel != 7)
+    return fail(c, WF_EINVAL, "kernel=%d must be 0 (default), 4 or 7", p->kernel);
+  for (int i = 0; i < 4; ++i)
     if (p->reserved[i]) return fail(c, WF_EINVAL, "reserved[%d] must be 0", i);
   if (p->alphabet < 0 || p->alphabet > 8) return fail(c, WF_EINVAL, "alphabet=%d out of range 0..8", p->alphabet);
   if (p->alphabet != 0 && p->fn != WF_FN_SEQCMP) return fail(c, WF_EINVAL, "alphabet applies to SEQCMP only");
@@ -147,11 +154,11 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
     default:
       return fail(c, WF_EINVAL, "fn=%d unknown", p->fn);
   }
-  defaults(*p, &pl.k, &pl.warps, &pl.skew);
+  defaults(*p, &pl.k, &pl.warps, &pl.skew, &pl.impl);
   if (pl.k != 1 && pl.k != 2 && pl.k != 4 && pl.k != 8) return fail(c, WF_EINVAL, "lane_cols=%d not in {1,2,4,8}", pl.k);
   if (pl.warps < 1 || pl.warps > 8) return fail(c, WF_EINVAL, "warps=%d out of range 1..8", pl.warps);
   if (pl.skew < 1 || pl.skew > 4) return fail(c, WF_EINVAL, "skew=%d out of range 1..4", pl.skew);
-  if (!wfk::variant_exists(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew))
+  if (!wfk::variant_exists(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew, pl.impl))
     return fail(c, WF_EUNSUPPORTED, "no kernel variant for fn=%d dsize=%d lane_cols=%d warps=%d skew=%d", p->fn,
                 p->dsize, pl.k, pl.warps, pl.skew);
   pl.band_w = p->fn == WF_FN_NASH ? pl.warps : pl.warps * 32 * pl.k;   // NASH: one column per warp
@@ -241,6 +248,7 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   c->c1 = pl.c1;
   c->k = pl.k;
   c->warps = pl.warps;
+  c->impl = pl.impl;
   c->skew = pl.skew;
   c->band_w = pl.band_w;
   c->nbands = pl.nbands;
@@ -268,6 +276,7 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   L.fn = p->fn;
   L.dsize = p->dsize;
   L.local = p->fn == WF_FN_SEQCMP ? p->local : 0;
+  L.impl = pl.impl;
   L.k = pl.k;
   L.warps = pl.warps;
   L.skew = pl.skew;
@@ -460,6 +469,7 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   L.tsize = p.tsize;
   L.dsize = p.dsize;
   L.local = p.fn == WF_FN_SEQCMP ? p.local : 0;
+  L.impl = c->impl;
   L.lane_best = c->lane_best;
   L.best_out = c->best_out;
   L.c0 = c->c0;

@@ -225,20 +225,23 @@ const Variant* table(size_t* n) {
   return v;
 }
 
-// SEQCMP at skew 1: the v4 kernel (block hand-offs) is the default -- measured faster on C4
-// (profiles/r01_nw7_experiments.txt); WF_NW_IMPL=7 selects the per-row hand-off v7 kernel
-bool want_nw7() {
+// Kernel generation (wf_params.kernel; the WF_NW_IMPL / WF_SYN_IMPL environment variables
+// override it for experiments).  SEQCMP at skew 1: v4 (block hand-offs) unless 7 is asked --
+// v4 measured faster on C4.
+bool want_nw7(int impl) {
   const char* e = getenv("WF_NW_IMPL");
-  return e && e[0] == '7';
+  if (e && e[0]) return e[0] == '7';
+  return impl == 7;
 }
 
-// SYNTHETIC at skew 1 runs the wf_syn.cu kernel unless WF_SYN_IMPL=4 (the generic sweep)
-bool want_syn7() {
+// SYNTHETIC at skew 1 runs the wf_syn.cu kernel unless generation 4 (the generic sweep) is asked
+bool want_syn7(int impl) {
   const char* e = getenv("WF_SYN_IMPL");
-  return !(e && e[0] == '4');
+  if (e && e[0]) return e[0] != '4';
+  return impl != 4;
 }
 
-const Variant* find(int fn, int dsize, int k, int warps, int skew) {
+const Variant* find(int fn, int dsize, int k, int warps, int skew, int impl) {
   size_t n;
   if (fn == WF_FN_SEQCMP && dsize == 1) {   // local alignment (Smith-Waterman)
     const Variant* ts = sw_table(&n);
@@ -246,12 +249,12 @@ const Variant* find(int fn, int dsize, int k, int warps, int skew) {
       if (ts[i].k == k && ts[i].warps == warps && ts[i].skew == skew) return &ts[i];
     return nullptr;
   }
-  if (fn == WF_FN_SEQCMP && skew == 1 && want_nw7()) {
+  if (fn == WF_FN_SEQCMP && skew == 1 && want_nw7(impl)) {
     const Variant* t7 = nw7_table(&n);
     for (size_t i = 0; i < n; ++i)
       if (t7[i].k == k && t7[i].warps == warps) return &t7[i];
   }
-  if (fn == WF_FN_SYNTHETIC && skew == 1 && want_syn7()) {
+  if (fn == WF_FN_SYNTHETIC && skew == 1 && want_syn7(impl)) {
     const Variant* t7 = syn_table(&n);
     for (size_t i = 0; i < n; ++i)   // a wf_syn variant whose staging rings do not fit falls back to the generic sweep
       if (t7[i].dsize == dsize && t7[i].k == k && t7[i].warps == warps && t7[i].smem <= 232448) return &t7[i];
@@ -264,21 +267,21 @@ const Variant* find(int fn, int dsize, int k, int warps, int skew) {
 
 }  // namespace
 
-bool variant_exists(int fn, int dsize, int k, int warps, int skew) {
+bool variant_exists(int fn, int dsize, int k, int warps, int skew, int impl) {
   // compiled AND within the 227 KB per-CTA shared-memory limit of sm_100
-  const Variant* v = find(fn, (fn == WF_FN_SYNTHETIC || fn == WF_FN_SEQCMP) ? dsize : 0, k, warps, skew);
+  const Variant* v = find(fn, (fn == WF_FN_SYNTHETIC || fn == WF_FN_SEQCMP) ? dsize : 0, k, warps, skew, impl);
   return v != nullptr && v->smem <= 232448;
 }
 
 int smem_bytes(const SweepLaunch& L) {
-  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew);
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew, L.impl);
   if (!v) return -1;
   if (L.fn == WF_FN_NASH) return (int)(v->smem + size_t(L.warps) * ((size_t(2) * L.tsize * L.tsize + 2 * L.tsize + 15) & ~size_t(15)));
   return (int)v->smem;
 }
 
 int occupancy(const SweepLaunch& L, int smem) {
-  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew);
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew, L.impl);
   if (!v) return 0;
   if (cudaFuncSetAttribute(v->kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem) != cudaSuccess) {
     cudaGetLastError();
@@ -293,7 +296,7 @@ int occupancy(const SweepLaunch& L, int smem) {
 }
 
 cudaError_t launch(const SweepLaunch& L, cudaStream_t s) {
-  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew);
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew, L.impl);
   if (!v) return cudaErrorInvalidDeviceFunction;
   return v->launch(L, s, (size_t)smem_bytes(L));
 }

@@ -38,10 +38,12 @@ import oracle  # noqa: E402  (parity gate only; the timed path never touches it)
 import workloads  # noqa: E402
 from paper_conf_ppopp_mohantyc14_b200.wf import Wavefront  # noqa: E402
 
+# impl = wf_params.kernel: 4 = first generation (NW v4 / generic synthetic sweep),
+# 7 = second generation (NW v7 / wf_syn); Nash has one kernel (0)
 SEARCH = {
-    "seqcmp": {"k": [2, 4, 8], "w": [1, 2, 4], "d": [1, 2], "impl": ["4", "7"]},
-    "synthetic": {"k": [1, 2], "w": [1, 2, 4], "d": [1, 2], "impl": ["syn7", "generic"]},
-    "nash": {"k": [1], "w": [1, 2, 4, 8], "d": [1], "impl": ["-"]},
+    "seqcmp": {"k": [2, 4, 8], "w": [1, 2, 4], "d": [1, 2], "impl": [4, 7]},
+    "synthetic": {"k": [1, 2], "w": [1, 2, 4], "d": [1, 2], "impl": [7, 4]},
+    "nash": {"k": [1], "w": [1, 2, 4, 8], "d": [1], "impl": [0]},
 }
 
 
@@ -82,20 +84,11 @@ def fn_kw(cfg):
     return dict(tsize=cfg.tsize, dsize=4)
 
 
-def set_impl(fn, impl):
-    os.environ.pop("WF_NW_IMPL", None)
-    os.environ.pop("WF_SYN_IMPL", None)
-    if fn == "seqcmp":
-        os.environ["WF_NW_IMPL"] = impl
-    elif fn == "synthetic" and impl == "generic":
-        os.environ["WF_SYN_IMPL"] = "4"
-
-
-def parity_ok(cfg, k, w, d, dev, small):
+def parity_ok(cfg, k, w, d, impl, dev, small):
     host, devin = inputs_for(cfg.fn, small, cfg.dsize, dev)
     small_cfg = workloads.Config(cfg.name, cfg.fn, small, tsize=cfg.tsize, dsize=cfg.dsize)
     want = oracle_grid(cfg.fn, host, small_cfg)
-    with Wavefront(cfg.fn, small, lane_cols=k, warps=w, skew=d, **fn_kw(cfg)) as wf:
+    with Wavefront(cfg.fn, small, lane_cols=k, warps=w, skew=d, kernel=impl, **fn_kw(cfg)) as wf:
         out = wf.run(*devin)
         wf.sync()
         got = [o.cpu().numpy() for o in out]
@@ -112,8 +105,8 @@ def parity_ok(cfg, k, w, d, dev, small):
     return True
 
 
-def time_point(cfg, k, w, d, devin, reps):
-    with Wavefront(cfg.fn, cfg.dim, lane_cols=k, warps=w, skew=d, **fn_kw(cfg)) as wf:
+def time_point(cfg, k, w, d, impl, devin, reps):
+    with Wavefront(cfg.fn, cfg.dim, lane_cols=k, warps=w, skew=d, kernel=impl, **fn_kw(cfg)) as wf:
         out = wf.alloc_out()
         for _ in range(3):
             wf.run(*devin, out=out)
@@ -137,24 +130,22 @@ def tune(cfg, reps, small, budget_s):
     points = []
     t_start = time.time()
     for impl, k, w, d in itertools.product(sp["impl"], sp["k"], sp["w"], sp["d"]):
-        if cfg.fn == "seqcmp" and impl == "7" and d != 1:
+        if cfg.fn == "seqcmp" and impl == 7 and d != 1:
             continue
         if time.time() - t_start > budget_s:
             points.append({"impl": impl, "k": k, "w": w, "d": d, "skipped": "time budget"})
             continue
-        set_impl(cfg.fn, impl)
         rec = {"impl": impl, "k": k, "w": w, "d": d}
         try:
-            if not parity_ok(cfg, k, w, d, dev, small):
+            if not parity_ok(cfg, k, w, d, impl, dev, small):
                 rec["error"] = "parity mismatch vs oracle"
             else:
-                ms, nb = time_point(cfg, k, w, d, devin, reps)
+                ms, nb = time_point(cfg, k, w, d, impl, devin, reps)
                 rec.update(ms=round(ms, 4), gcups=round(cfg.dim * cfg.dim / ms / 1e6, 3), nbands=nb)
         except Exception as e:  # noqa: BLE001 -- unsupported variants are part of the sweep
             rec["error"] = str(e)[:160]
         points.append(rec)
         print(json.dumps(rec), flush=True)
-    set_impl(cfg.fn, "")
     ok = [p for p in points if "ms" in p]
     best = min(ok, key=lambda p: p["ms"]) if ok else None
     return {"config": cfg.name, "workload": cfg.note or cfg.name, "fn": cfg.fn, "dim": cfg.dim, "tsize": cfg.tsize,
@@ -162,8 +153,40 @@ def tune(cfg, reps, small, budget_s):
             "parity_dim": small, "reps": reps, "best": best, "points": points}
 
 
+# Problem design for the learned tuner (tools/train_tuner.py): the
+# paper trained its models on sweeps over (dim, tsize, dsize); here the
+# same features on B200 sizes.
+GRID = ([("seqcmp", d, 0, 0) for d in (1024, 2048, 4096, 8192, 16384, 32768)]
+        + [("synthetic", d, t, ds) for d in (1024, 4096, 16384) for t in (10, 100, 1000) for ds in (1, 3, 5)]
+        + [("nash", d, 16, 4) for d in (1024, 2048, 4096)])
+
+
+def sweep_grid(reps, out):
+    dev = torch.device("cuda", 0)
+    recs = []
+    for fn, dim, tsize, dsize in GRID:
+        cfg = workloads.Config(f"{fn}-{dim}-{tsize}-{dsize}", fn, dim, tsize=tsize, dsize=dsize)
+        _, devin = inputs_for(fn, dim, dsize, dev)
+        sp = SEARCH[fn]
+        for impl, k, w, d in itertools.product(sp["impl"], sp["k"], sp["w"], sp["d"]):
+            if fn == "seqcmp" and impl == 7 and d != 1:
+                continue
+            rec = {"fn": fn, "dim": dim, "tsize": tsize, "dsize": dsize, "impl": impl, "k": k, "w": w, "d": d}
+            try:
+                ms, nb = time_point(cfg, k, w, d, impl, devin, reps)
+                rec.update(ms=round(ms, 5), nbands=nb)
+            except Exception as e:  # noqa: BLE001
+                rec["error"] = str(e)[:120]
+            recs.append(rec)
+            print(json.dumps(rec), flush=True)
+        del devin
+    with open(out, "w") as f:
+        json.dump({"device": torch.cuda.get_device_name(0), "reps": reps, "points": recs}, f, indent=0)
+
+
 def main():
     ap = argparse.ArgumentParser()
+    ap.add_argument("--grid", action="store_true", help="sweep the tuner's problem design (GRID)")
     ap.add_argument("--config", default="C5a", choices=sorted(workloads.CONFIGS))
     ap.add_argument("--all", action="store_true")
     ap.add_argument("--reps", type=int, default=5)
@@ -171,6 +194,9 @@ def main():
     ap.add_argument("--budget-s", type=float, default=240.0, help="per-config time budget")
     ap.add_argument("--out", default="")
     a = ap.parse_args()
+    if a.grid:
+        sweep_grid(a.reps, a.out or os.path.join(ROOT, "profiles", "tuner_sweep.json"))
+        return
     names = sorted(workloads.CONFIGS) if a.all else [a.config]
     for n in names:
         cfg = workloads.CONFIGS[n]
