@@ -158,6 +158,10 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   if (pl.k != 1 && pl.k != 2 && pl.k != 4 && pl.k != 8) return fail(c, WF_EINVAL, "lane_cols=%d not in {1,2,4,8}", pl.k);
   if (pl.warps < 1 || pl.warps > 8) return fail(c, WF_EINVAL, "warps=%d out of range 1..8", pl.warps);
   if (pl.skew < 1 || pl.skew > 4) return fail(c, WF_EINVAL, "skew=%d out of range 1..4", pl.skew);
+  // a default band width whose shared-memory rings do not fit (many planes) halves until it does
+  while (!p->warps && pl.warps > 1 &&
+         !wfk::variant_exists(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew, pl.impl))
+    pl.warps /= 2;
   if (!wfk::variant_exists(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew, pl.impl))
     return fail(c, WF_EUNSUPPORTED, "no kernel variant for fn=%d dsize=%d lane_cols=%d warps=%d skew=%d", p->fn,
                 p->dsize, pl.k, pl.warps, pl.skew);

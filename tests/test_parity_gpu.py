@@ -238,6 +238,34 @@ def test_seqcmp_c4_full_grid():
     assert np.array_equal(H, g)
 
 
+@pytest.mark.parametrize("kind,scoring", [("identical", (1, -1, -1)), ("disjoint", (1, -1, -1)),
+                                          ("disjoint", (1, -1, -2))])
+def test_seqcmp_maximum_dim_closed_forms(kind, scoring):
+    """dim = 65535 (the ABI maximum; 4.3 G cells, 17 GB of output): closed forms of the
+    recurrence checked on sampled rows -- identical sequences H = min(i,j) M + |i-j| G;
+    disjoint alphabets H = min(i,j) X + |i-j| G when X >= 2G (else -max(i,j) for (1,-1,-1))."""
+    dim = 65535
+    x, y = workloads.seqcmp_inputs(dim, dim, kind=kind)
+    M, X, G = scoring
+    dev = torch.device("cuda", torch.cuda.current_device())
+    with Wavefront("seqcmp", dim, match=M, mismatch=X, gap=G, alphabet=4) as w:
+        row_in, col_in, top, left = dev_inputs("seqcmp", (x, y), dev)
+        (g,) = w.run(row_in, col_in, top, left)
+        w.sync()
+        j = np.arange(1, dim + 1, dtype=np.int64)
+        for i in (1, 2, 31, 32, 33, 1000, 32767, 32768, 65534, 65535):
+            row = g[i - 1].cpu().numpy().astype(np.int64)
+            lo, d = np.minimum(i, j), np.abs(i - j)
+            if kind == "identical":
+                want = lo * M + d * G
+            elif X >= 2 * G:
+                want = lo * X + d * G
+            else:
+                want = -np.maximum(i, j)
+            assert np.array_equal(row, want), (kind, scoring, i)
+        del g
+
+
 # ------------------------------------------------------------------ synthetic
 def _syn(dim, tsize, dsize, cols=0, seeds=(3, 4, 5), m_compute=None, **kw):
     n = cols or dim
