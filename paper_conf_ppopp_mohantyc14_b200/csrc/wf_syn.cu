@@ -29,7 +29,16 @@
 namespace wfk {
 
 constexpr int kSynLL = 128;   // rows per shared west LL ring (power of 2)
-constexpr int kSynU = 16;     // rows per TMA write-back block
+// Block sizes, measured on C2 / C5a-c:
+//  * TMA write-back window UT: 32 rows amortise the proxy fence; 16 rows when the planes are
+//    many (dsize > 2), so that 4 one-warp CTAs still fit per SM (512 bands at dim 16384).
+//  * west hand-off block UB: the hand-off lag is UB + 31 steps per warp; with deep cells
+//    (large tsize) a step is expensive and small blocks win, with light cells the per-block
+//    cost dominates: UB = 16 / 8 / 4 for tsize x dsize < 40 / < 1000 (or runtime) / >= 1000.
+__host__ __device__ constexpr int syn_ut(int ds) { return ds <= 2 ? 32 : 16; }
+__host__ __device__ constexpr int syn_ub(int ts, int ds) {
+  return ts == 0 ? 8 : (ts * (ds > 0 ? ds : 1) >= 1000 ? 4 : ts * (ds > 0 ? ds : 1) >= 40 ? 8 : 16);
+}
 
 struct SynMaps {
   CUtensorMap m[WF_MAX_PLANES];
@@ -39,8 +48,10 @@ template <int DS, int K, int WARPS>
 struct SynSmem {
   static constexpr int NF = 2 + DS;         // output planes / west words per row
   static constexpr int NWD = NF + 1;        // + the row input u_i
-  static constexpr int U = kSynU;
-  static constexpr int R = 64;              // staging rows alive: skew 31 + block U + TMA block U
+  static constexpr int U = syn_ut(DS);
+  // staging rows alive: skew 31 + the TMA window being filled + the window whose TMA store
+  // may still be reading
+  static constexpr int R = (2 * U + 31) <= 64 ? 64 : 128;
   static_assert(2 * U + 31 <= R, "staging ring too small");
   static constexpr int ROWB = 32 * K * 4;
   static constexpr size_t stage_bytes = size_t(WARPS) * NF * R * ROWB;
@@ -216,7 +227,7 @@ struct SynWarp {
     uint32_t* nring = LAST ? nullptr : sm.ll + size_t(warp + 1) * kSynLL * NWD;
     const bool glob = LAST && gdst != nullptr;
 #pragma unroll
-    for (int u = 0; u < U; ++u) {
+    for (int u = 0; u < syn_ub(TS, DS); ++u) {
       const int t = t0 + u;
       const int row = t - lane + 1;
       uint32_t Win[NF];
@@ -290,15 +301,19 @@ struct SynWarp {
 #pragma unroll
     for (int f = 0; f < NF; ++f) q[f] = 0u;
     const uint32_t stage_s = static_cast<uint32_t>(__cvta_generic_to_shared(stage_w));
-    for (int t0 = 0; t0 < T; t0 += U) {
-      // this block reads rows t0+2 .. t0+U+1 of my ring (row t0+1 is already in pre)
-      if (!wait_ctr(sm.wprog + warp, min(t0 + U + 1, rows), seen_w)) return false;
+    constexpr int UB = syn_ub(TS, DS);
+    static_assert(U % UB == 0, "hand-off blocks tile the write-back window");
+    for (int t0 = 0; t0 < T; t0 += UB) {
+      // this block reads rows t0+2 .. t0+UB+1 of my ring (row t0+1 is already in pre)
+      if (!wait_ctr(sm.wprog + warp, min(t0 + UB + 1, rows), seen_w)) return false;
       if (lane == 0) sts_vol_i(sm.rprog + warp, t0 + 1);   // rows <= t0+1 of my ring consumed
-      // lane 31 writes rows t0-30 .. t0-31+U into the next ring: their slots must be free
-      if (!last && !wait_ctr(sm.rprog + warp + 1, t0 - 31 + U - kSynLL, seen_r)) return false;
-      if (lane == 0) bulk_wait_read<1>();                  // staging slots of 2 blocks ago are free
-      __syncwarp();
-      const bool steady = t0 >= 32 && t0 + U + 1 <= rows;
+      // lane 31 writes rows t0-30 .. t0-31+UB into the next ring: their slots must be free
+      if (!last && !wait_ctr(sm.rprog + warp + 1, t0 - 31 + UB - kSynLL, seen_r)) return false;
+      if (t0 % U == 0) {
+        if (lane == 0) bulk_wait_read<1>();                // staging slots of 2 windows ago are free
+        __syncwarp();
+      }
+      const bool steady = t0 >= 32 && t0 + UB + 1 <= rows;
       if (last) {
         if (steady) block<false, true>(t0, pre, q, qx, gdst, to_peer);
         else block<true, true>(t0, pre, q, qx, gdst, to_peer);
@@ -307,14 +322,17 @@ struct SynWarp {
         else block<true, false>(t0, pre, q, qx, gdst, to_peer);
       }
       // publish lane 31's rows of the block to the next warp (one fence per block)
-      const int r31_0 = t0 - 30;
-      const int r31_last = min(r31_0 + U - 1, rows);
+      const int r31_last = min(t0 + UB - 31, rows);
       if (!last && r31_last >= 1 && lane == 31) {
         __threadfence_block();
         sts_vol_i(sm.wprog + warp + 1, r31_last);
       }
-      // write back lane 31's rows of the block (every lane is past them)
-      if (r31_last >= 1) {
+      // write back lane 31's rows of the U-row window (every lane is past them): one TMA box
+      // per plane when the window is complete (or the sweep ends)
+      const bool win_end = (t0 + UB) % U == 0 || t0 + UB >= T;
+      if (win_end && r31_last >= 1) {
+        const int w0 = ((t0 + UB - 1) / U) * U;            // window start step (multiple of U)
+        const int r31_0 = w0 - 30;                          // its first lane-31 row
         fence_proxy_async_smem();
         __syncwarp();
         if (r31_0 >= 1) {
@@ -447,7 +465,7 @@ cudaError_t launch_syn(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   SynMaps maps;
   memset(&maps, 0, sizeof maps);
   for (int f = 0; f < 2 + DS; ++f) {
-    cudaError_t e = encode_plane_map_f(&maps.m[f], L, f, 32 * K, kSynU);
+    cudaError_t e = encode_plane_map_f(&maps.m[f], L, f, 32 * K, syn_ut(DS));
     if (e != cudaSuccess) return e;
   }
   // tsize of the BASELINE configs (10, 100, 1000) as a compile-time trip count for the
@@ -477,7 +495,7 @@ Variant make_syn() {
 
 const Variant* syn_table(size_t* n) {
 #ifdef WF_MIN_VARIANTS
-  static const Variant v[] = {WF_SYN7(1)};
+  static const Variant v[] = {WF_SYN7(1), WF_SYN7(5)};
 #else
   static const Variant v[] = {WF_SYN7(0), WF_SYN7(1), WF_SYN7(2), WF_SYN7(3), WF_SYN7(4),
                               WF_SYN7(5), WF_SYN7(6), WF_SYN7(7), WF_SYN7(8)};
