@@ -117,21 +117,24 @@ __device__ __forceinline__ void nash_solve16(uint32_t key, int lane, uint32_t o[
 #pragma unroll
     for (int q = 0; q < 4; ++q) P[q] = __vmaxu2(P[q], __shfl_xor_sync(0xffffffffu, P[q], s));
   }
-  // ballots are warp-uniform, so the first non-empty one is picked with plain selects (no
-  // shuffles under a branch) and its payoffs fetched with one shuffle each afterwards
-  int count = 0, first = -1, src = 0;
-  uint32_t selA = 0, selB = 0;
+  // pure equilibria of the lane's 8 entries as a bit mask, then two warp reductions (REDUX):
+  // the count, and the smallest row-major index 32k + lane holding one (the first
+  // equilibrium); its payoffs come from the lane that owns it (one shuffle each)
+  uint32_t mask = 0, kmin = 8, selA = 0, selB = 0;
 #pragma unroll
-  for (int k = 0; k < 8; ++k) {
+  for (int k = 7; k >= 0; --k) {   // descending: the selects end on the smallest k
     const uint32_t rB = (k & 1) ? (P[k >> 1] >> 16) : (P[k >> 1] & 0xFFFFu);
-    const unsigned bal = __ballot_sync(0xffffffffu, A[k] == cA && B[k] == rB);
-    count += __popc(bal);
-    const bool take = first < 0 && bal != 0u;
-    src = take ? __ffs(bal) - 1 : src;
-    first = take ? 32 * k + src : first;
-    selA = take ? A[k] : selA;
-    selB = take ? B[k] : selB;
+    const bool ne = A[k] == cA && B[k] == rB;
+    mask |= ne ? (1u << k) : 0u;
+    kmin = ne ? static_cast<uint32_t>(k) : kmin;
+    selA = ne ? A[k] : selA;
+    selB = ne ? B[k] : selB;
   }
+  const int count = static_cast<int>(__reduce_add_sync(0xffffffffu, static_cast<unsigned>(__popc(mask))));
+  const uint32_t mine = mask ? 32u * kmin + static_cast<uint32_t>(lane) : 0xFFFFFFFFu;
+  const uint32_t firstu = __reduce_min_sync(0xffffffffu, mine);
+  const int first = firstu == 0xFFFFFFFFu ? -1 : static_cast<int>(firstu);
+  const int src = first < 0 ? 0 : (first & 31);
   uint32_t pa = __shfl_sync(0xffffffffu, selA, src);
   uint32_t pb = __shfl_sync(0xffffffffu, selB, src);
   if (first < 0) pa = pb = 0xFFFFFFFFu;
