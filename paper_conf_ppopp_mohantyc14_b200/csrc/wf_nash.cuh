@@ -58,6 +58,10 @@ struct PolNash {
 
 // Shared memory: inbound LL rings (one per warp), consumption counters, and per-warp
 // game scratch (A, B as bytes, column maxima of A, row maxima of B).
+#ifndef WF_NASH_REDUX_ROWMAX
+#define WF_NASH_REDUX_ROWMAX 0   // 1: row maxima of B by half-warp REDUX instead of a shuffle butterfly
+#endif
+
 template <int WARPS>
 struct NashSmem {
   static constexpr int kSlots = 128;                                        // rows per ring
@@ -110,6 +114,13 @@ __device__ __forceinline__ void nash_solve16(uint32_t key, int lane, uint32_t o[
   // row maxima of B: row (l >> 4) + 2k spans the 16 lanes of the half -> butterfly over
   // xor 1, 2, 4, 8 on two rows at a time (16-bit SIMD max)
   uint32_t P[4];
+#if WF_NASH_REDUX_ROWMAX
+  // each half-warp is one group of the reduction (row (l >> 4) + 2k lives in one half)
+  const unsigned half = (lane < 16) ? 0x0000FFFFu : 0xFFFF0000u;
+#pragma unroll
+  for (int q = 0; q < 4; ++q)
+    P[q] = __reduce_max_sync(half, B[2 * q]) | (__reduce_max_sync(half, B[2 * q + 1]) << 16);
+#else
 #pragma unroll
   for (int q = 0; q < 4; ++q) P[q] = B[2 * q] | (B[2 * q + 1] << 16);
 #pragma unroll
@@ -117,6 +128,7 @@ __device__ __forceinline__ void nash_solve16(uint32_t key, int lane, uint32_t o[
 #pragma unroll
     for (int q = 0; q < 4; ++q) P[q] = __vmaxu2(P[q], __shfl_xor_sync(0xffffffffu, P[q], s));
   }
+#endif
   // pure equilibria of the lane's 8 entries as a bit mask, then two warp reductions (REDUX):
   // the count, and the smallest row-major index 32k + lane holding one (the first
   // equilibrium); its payoffs come from the lane that owns it (one shuffle each)
