@@ -243,7 +243,7 @@ def run_reference(args, cfg):
     value = rows * cfg.dim * args.steps / tot / 1e9
     line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": tot / args.steps * 1e3, "higher_is_better": True,
-            "scaling": "weak", "vs_baseline": None, "dtype": dtype_of(cfg), "data": "synthetic",
+            "scaling": "strong", "vs_baseline": None, "dtype": dtype_of(cfg), "data": "synthetic",
             "impl": "reference",
             "config": {"workload": cfg.name + ": " + cfg.note, "fn": cfg.fn, "dim": cfg.dim, "tsize": cfg.tsize,
                        "dsize": cfg.dsize, "sample_rows": rows},
@@ -394,7 +394,7 @@ def run_ours(args, cfg):
     if rank == 0:
         result = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
-            "warmup": args.warmup, "ms_per_step": step_ms, "higher_is_better": True, "scaling": "weak" if False else "strong",
+            "warmup": args.warmup, "ms_per_step": step_ms, "higher_is_better": True, "scaling": "strong",
             "vs_baseline": None, "dtype": dtype_of(cfg), "data": "synthetic (seeded PCG64 inputs, workloads/)",
             "config": {"workload": cfg.name + ": " + cfg.note, "fn": cfg.fn, "dim": cfg.dim, "tsize": cfg.tsize,
                        "dsize": cfg.dsize, "lane_cols": lay.lane_cols, "warps": lay.warps, "skew": lay.skew,

@@ -84,11 +84,13 @@ typedef struct {
   int32_t lane_cols;    /* tunable k: adjacent columns owned by one lane (1, 2, 4, 8); 0 = default */
   int32_t warps;        /* tunable: compute warps per CTA = column groups per band (1..8); 0 = default */
   int32_t skew;         /* tunable d: row lag between neighbouring lanes (1..4); 0 = default */
-  int32_t strip;        /* tunable: rows per inter-slab message (NCCL transport); 0 = default */
+  int32_t strip;        /* rows per inter-slab message of a strip transport: must be 0 (the P2P
+                           transport hands off every row; > 0 -> WF_EUNSUPPORTED) */
   int32_t ngpus;        /* slabs (column blocks), 1..8; see wf_dist */
   int32_t match, mismatch, gap;  /* SEQCMP scores, each in [-64, 64]; defaults used if all three 0 */
   int32_t local;        /* SEQCMP: 0 = global (Needleman-Wunsch), 1 = local (Smith-Waterman) */
-  uint32_t transport;   /* wf_transport for ngpus > 1 */
+  uint32_t transport;   /* wf_transport for ngpus > 1: only WF_TRANSPORT_P2P is built; NCCL ->
+                           WF_EUNSUPPORTED */
   uint32_t max_ctas;    /* 0 = all resident CTAs; else an upper bound (tests of the band loop) */
   uint64_t watchdog_cycles; /* spin budget per dependency wait (SM clock cycles); 0 = default 2^32 */
   int32_t alphabet;     /* SEQCMP: 0 = residue codes may be any byte value; 1..8 = every code in

@@ -117,7 +117,14 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   const int G = p->ngpus ? p->ngpus : 1;
   if (rank < 0 || rank >= G) return fail(c, WF_EINVAL, "rank=%d out of range for ngpus=%d", rank, G);
   if (p->transport > WF_TRANSPORT_NCCL) return fail(c, WF_EINVAL, "transport=%u unknown", p->transport);
+  // The slab hand-off is per-row P2P LL words stored by the sweep itself; the
+  // host-driven NCCL strip exchange and its strip size are not built, and are refused rather
+  // than silently ignored.
+  if (p->transport == WF_TRANSPORT_NCCL)
+    return fail(c, WF_EUNSUPPORTED, "transport=NCCL is not built (P2P per-row hand-off only, DESIGN.md §8)");
   if (p->strip < 0) return fail(c, WF_EINVAL, "strip=%d must be >= 0", p->strip);
+  if (p->strip > 0)
+    return fail(c, WF_EUNSUPPORTED, "strip=%d: the P2P transport hands off every row; strip must be 0", p->strip);
   if (p->lane_cols < 0 || p->warps < 0 || p->skew < 0)
     return fail(c, WF_EINVAL, "lane_cols/warps/skew must be >= 0");
   Plan pl{};

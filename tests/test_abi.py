@@ -68,6 +68,14 @@ def test_query_rejects_bad_params_naming_the_field(kw, field):
     assert field in str(e)
 
 
+@pytest.mark.parametrize("kw,field", [(dict(transport="nccl"), "transport"), (dict(strip=256), "strip")])
+def test_unbuilt_transport_options_are_refused(kw, field):
+    # the slab hand-off is the sweep's own per-row P2P store; the NCCL strip
+    # transport is not built and must not be accepted and silently ignored
+    e = _err("seqcmp", 256, ngpus=2, **kw)
+    assert e.status == _abi.WF_EUNSUPPORTED and field in str(e)
+
+
 def test_reserved_fields_must_be_zero():
     p = make_params("seqcmp", 64)
     p.reserved[2] = 1
