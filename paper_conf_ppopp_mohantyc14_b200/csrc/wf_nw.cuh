@@ -331,7 +331,10 @@ struct NwWarp {
         return true;
       }
       if (wd.expired(L)) return false;
-      __nanosleep(sleep_ns);
+#ifndef WF_NW_WAIT_SLEEP
+#define WF_NW_WAIT_SLEEP 1     // 0: compute warps spin on shared counters without back-off
+#endif
+      if (WF_NW_WAIT_SLEEP) __nanosleep(sleep_ns);
     }
   }
 
@@ -482,13 +485,33 @@ struct NwWarp {
         tc = n;
       }
     };
-    for (; t0 < T; t0 += U, ++blk) {
+    // Instruction-cache warm-up (WF_NW_WARM): the steady and edge block bodies are ~100 KB of
+    // unrolled SASS, and every band's first pass through them was paying the misses on the
+    // band-to-band critical path.  A band that waits for its west input anyway first runs one
+    // steady and one edge block through the SAME call site on dummy inputs (their staging
+    // stores land in slots that real rows overwrite before any publish), then restores the
+    // lane state.  Band 0 of the first slab starts at once and skips it.
+#ifndef WF_NW_WARM
+#define WF_NW_WARM 1
+#endif
+    int warm = (WF_NW_WARM && !(L.first_slab && band == 0)) ? 2 : 0;
+    int32_t sv_Np[K], sv_q[D];
+    uint32_t sv_xq[D];
+    const int32_t sv_prevW = prevW, sv_best = best, sv_best_row = best_row;
+#pragma unroll
+    for (int m = 0; m < K; ++m) sv_Np[m] = Np[m];
+#pragma unroll
+    for (int d = 0; d < D; ++d) {
+      sv_q[d] = q[d];
+      sv_xq[d] = xq[d];
+    }
+    for (; t0 < T;) {
       const int r0 = t0 + 1;                       // lane 0's first row in this block
       const int rl = min(t0 + U, rows);            // its last valid row
       // ---- west inputs and row codes of lane 0's rows r0 .. r0+U-1: one shared load each
       int32_t wv = 0;
       uint32_t xv = 0;
-      if (rl >= 1) {
+      if (!warm && rl >= 1) {
         if (!wait_ctr(wprog_src, rl, seen_wprog, 20)) return false;
         if (!wait_ctr(sm.xfill, rl, seen_xfill, 32)) return false;
         tick(0);
@@ -500,7 +523,7 @@ struct NwWarp {
       }
       // rows < r0 of the source are no longer needed (the loads above are complete once
       // used; publish one block late to be safe)
-      if (lane == 0 && blk > 0) {
+      if (!warm && lane == 0 && blk > 0) {
         sts_vol_i(rprog_src, r0 - U - 1 + U);
         sts_vol_i(sm.xneed + warp, r0);
       }
@@ -508,18 +531,34 @@ struct NwWarp {
       // ---- my staging ring: slots of rows <= lane 0's rows of this block minus R must be
       //      free: read by TMA (bulk groups) and by my reader (rprog[warp])
       const int need_free = t0 + U - R;
-      if (need_free >= 1) {
+      if (!warm && need_free >= 1) {
         if (lane == 0) bulk_wait_read<1>();
         __syncwarp();
         if (!wait_ctr(sm.rprog + warp, need_free, seen_rprog, 20)) return false;
       }
       tick(2);
       int32_t east_last;
-      if (L.trace && lane == 0 && t0 <= steady_lo && t0 + U > steady_lo)   // entering steady state
+      if (!warm && L.trace && lane == 0 && t0 <= steady_lo && t0 + U > steady_lo)   // entering steady state
         L.trace[size_t(band) * kTraceSlots + 33 + warp] = globaltimer();
-      if (t0 >= steady_lo && t0 <= steady_hi) block<false>(t0, wv, xv, east_last);
-      else block<true>(t0, wv, xv, east_last);
+      const int tb = warm == 2 ? steady_lo : warm == 1 ? -4 * U : t0;   // block start step
+      if (tb >= steady_lo && tb <= steady_hi) block<false>(tb, wv, xv, east_last);
+      else block<true>(tb, wv, xv, east_last);
       (void)east_last;
+      if (warm) {
+        if (--warm == 0) {   // restore the lane state the dummy blocks advanced
+          prevW = sv_prevW;
+          best = sv_best;
+          best_row = sv_best_row;
+#pragma unroll
+          for (int m = 0; m < K; ++m) Np[m] = sv_Np[m];
+#pragma unroll
+          for (int d = 0; d < D; ++d) {
+            q[d] = sv_q[d];
+            xq[d] = sv_xq[d];
+          }
+        }
+        continue;
+      }
       tick(3);
       // ---- publish: one fence for the TMA engine and for the next warp
       const int r31_0 = t0 - 31 * D + 1;           // first row of the block's TMA box
@@ -533,11 +572,24 @@ struct NwWarp {
             bulk_commit();
           }
         } else {
+#ifndef WF_NW_EARLY_PUB
+#define WF_NW_EARLY_PUB 1
+#endif
+          // first block: publish before the generic-store write-back (the reader only needs the
+          // staging ring, fenced above, and these slots are not reused before row R), so the
+          // next warp's start does not wait for 32 rows of STGs
+          if (WF_NW_EARLY_PUB && lane == 0) sts_vol_i(sm.wprog + warp, r31_last);
           for (int r = 1; r <= r31_last; ++r) write_row(r);
         }
         if (lane == 0) sts_vol_i(sm.wprog + warp, r31_last);
       }
       tick(4);
+#ifdef WF_NW_TRACE_BLOCKS   // ramp cadence: end of the first 15 blocks (perturbs the code layout)
+      if (L.trace && lane == 0 && warp < 2 && blk < 15)
+        L.trace[size_t(band) * kTraceSlots + 1 + 15 * warp + blk] = globaltimer();
+#endif
+      t0 += U;
+      ++blk;
     }
     if (prof)
       for (int i = 0; i < 5; ++i) L.trace[size_t(band) * kTraceSlots + 48 + 5 * warp + i] = ph[i];
@@ -583,6 +635,22 @@ __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K,
     r_wprog = dsmem_addr(sm.wprog + WARPS, crank + 1);
     r_rprog = dsmem_addr(sm.rprog + WARPS, crank + 1);
   }
+  // I/O warp back-off (ns) after a productive / idle pass.  With WARPS <= 2 the I/O warp
+  // (warp WARPS) has an SM sub-partition of its own, so it spins without sleeping: measured
+  // C4 2.718 -> 2.659 ms (profiles/r01_io_spin_ab.txt).  Otherwise it shares a scheduler with
+  // compute warp 0 and backs off.
+#ifndef WF_NW_IO_NS_BUSY
+#define WF_NW_IO_NS_BUSY (WARPS <= 2 ? 0 : 64)
+#endif
+#ifndef WF_NW_IO_NS_IDLE
+#define WF_NW_IO_NS_IDLE (WARPS <= 2 ? 0 : 128)
+#endif
+#ifndef WF_NW_LL_GPU
+#define WF_NW_LL_GPU 0         // 1: band-to-band rings on this device use .gpu-scope LL accesses
+#endif
+  // the inbound ring is written by this device unless it is band 0 of a slab g > 0 (peer GPU)
+  const bool src_local = WF_NW_LL_GPU && band > 0;
+  const bool dst_local = WF_NW_LL_GPU && band + 1 < L.nbands;
   int feed = from_cluster ? rows + 1 : 1;   // next row to feed (the producer feeds a cluster band)
   int fwd = 1;                  // next row to forward from the last warp's staging ring
   int seen_feed_rd = 0, seen_last_wr = 0, seen_remote_rd = 0;
@@ -607,7 +675,7 @@ __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K,
             if (boundary) {
               v[h] = LOCAL ? 0 : r * L.gap;                       // H[r][0] = r*g (NW), 0 (SW)
             } else {
-              const unsigned long long wv = ld_relaxed_sys(src + r);
+              const unsigned long long wv = src_local ? ld_relaxed_gpu(src + r) : ld_relaxed_sys(src + r);
               v[h] = static_cast<int32_t>(static_cast<uint32_t>(wv));
               ok[h] = static_cast<uint32_t>(wv >> 32) == L.epoch;
             }
@@ -658,6 +726,7 @@ __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K,
           if (lane < n) {
             const int32_t v = lds_vol_s32(east_col + ((r + last_off) & (S::R - 1)) * S::ROWB);
             if (to_cluster) st_cluster_u32(r_feed + 4u * (r & (kFeed - 1)), static_cast<uint32_t>(v));
+            else if (dst_local) st_relaxed_gpu(dst + r, ll_pack(static_cast<uint32_t>(v), L.epoch));
             else if (dst) st_relaxed_sys(dst + r, ll_pack(static_cast<uint32_t>(v), L.epoch));
           }
           __syncwarp();   // orders every lane's DSMEM store before lane 0's release of the counter
@@ -672,10 +741,10 @@ __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K,
     }
     if (progress) {
       wd.start();
-      __nanosleep(64);
+      if (WF_NW_IO_NS_BUSY) __nanosleep(WF_NW_IO_NS_BUSY);
     } else {
       if (wd.expired(L)) return false;
-      __nanosleep(128);
+      if (WF_NW_IO_NS_IDLE) __nanosleep(WF_NW_IO_NS_IDLE);
     }
   }
   return true;

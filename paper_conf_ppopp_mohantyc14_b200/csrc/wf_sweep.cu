@@ -206,13 +206,13 @@ Variant make_nash_variant() {
 
 const Variant* table(size_t* n) {
 #ifdef WF_MIN_VARIANTS   // quick experimental builds (tools/ablate.sh)
-  static const Variant v[] = {WF_SEQ(4, 1, 1), WF_SEQ(4, 1, 2), WF_SEQ(4, 2, 1), WF_SEQ(2, 1, 1), WF_SEQ(8, 1, 1),
+  static const Variant v[] = {WF_SEQ(4, 1, 1), WF_SEQ(4, 1, 2), WF_SEQ(4, 2, 1), WF_SEQ(4, 3, 1), WF_SEQ(2, 1, 1), WF_SEQ(8, 1, 1),
                               WF_NASH(8), WF_NASH(2)};
 #else
   static const Variant v[] = {
       WF_SEQ(2, 1, 1), WF_SEQ(2, 2, 1), WF_SEQ(2, 4, 1), WF_SEQ(2, 1, 2), WF_SEQ(2, 2, 2), WF_SEQ(2, 4, 2),
       WF_SEQ(2, 2, 3), WF_SEQ(2, 4, 3),
-      WF_SEQ(4, 1, 1), WF_SEQ(4, 2, 1), WF_SEQ(4, 4, 1), WF_SEQ(4, 1, 2), WF_SEQ(4, 2, 2), WF_SEQ(4, 4, 2),
+      WF_SEQ(4, 1, 1), WF_SEQ(4, 2, 1), WF_SEQ(4, 3, 1), WF_SEQ(4, 4, 1), WF_SEQ(4, 1, 2), WF_SEQ(4, 2, 2), WF_SEQ(4, 4, 2),
       WF_SEQ(4, 1, 3), WF_SEQ(4, 2, 3),
       WF_SEQ(8, 1, 1), WF_SEQ(8, 2, 1), WF_SEQ(8, 1, 2), WF_SEQ(8, 2, 2),
       WF_SEQ(1, 1, 1), WF_SEQ(1, 2, 1), WF_SEQ(1, 4, 1),

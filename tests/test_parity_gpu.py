@@ -43,7 +43,7 @@ def test_seqcmp_dims_default_tiling(dim):
     assert np.array_equal(H, g)
 
 
-SEQ_VARIANTS = [(1, 1, 1), (1, 4, 1), (2, 1, 1), (2, 2, 2), (2, 2, 3), (2, 4, 1), (4, 1, 1), (4, 2, 1), (4, 1, 2),
+SEQ_VARIANTS = [(1, 1, 1), (1, 4, 1), (2, 1, 1), (2, 2, 2), (2, 2, 3), (2, 4, 1), (4, 1, 1), (4, 2, 1), (4, 3, 1), (4, 1, 2),
                 (4, 1, 3), (8, 1, 1), (8, 1, 2)]
 
 

@@ -105,6 +105,10 @@ def main():
                                                         for w in range(min(4, wf.layout.warps))],
                     "feeder_polls": [int(x) for x in tr[:: max(1, len(tr) // 8), 40]],
                     "feeder_empty": [int(x) for x in tr[:: max(1, len(tr) // 8), 41]],
+                    # NW: end of the first 15 blocks of warps 0 / 1, us after the band's feed of 32 rows
+                    "nw_block_ends_us_band1": [[round(float(tr[1, 1 + 15 * w + b] - tr[1, 37]) / 1e3, 2)
+                                                for b in range(15)] for w in range(min(2, wf.layout.warps))]
+                    if len(tr) > 1 else [],
                     "raw32_band0": [int(x) for x in tr[0, 32:64]],
                     "raw32_mid": [int(x) for x in tr[len(tr) // 2, 32:64]],
                 })
