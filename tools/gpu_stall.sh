@@ -7,5 +7,6 @@ for c in C4 C5a; do
   ncu -i gpurun_out/st_$c.ncu-rep --page source --csv --print-source sass > gpurun_out/st_${c}_sass.csv 2>/dev/null
   ncu -i gpurun_out/st_$c.ncu-rep --page source --csv --print-source cuda,sass > gpurun_out/st_${c}_cs.csv 2>/dev/null
   ncu -i gpurun_out/st_$c.ncu-rep --page source --csv --print-source cuda > gpurun_out/st_${c}_cuda.csv 2>/dev/null
+  rm -f gpurun_out/st_$c.ncu-rep
 done
 ls -la gpurun_out/st_*
