@@ -427,8 +427,19 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
   return true;
 }
 
+// Idle warps appended to each CTA: they only join the band barriers.  With one compute warp +
+// one feeder per CTA, consecutive CTAs of an SM place their compute warps on the same SM
+// sub-partitions; a CTA of 2 + 2 warps moves the next CTA's compute warp to another one.
+// Measured (interleaved A/B, one-warp variant): dsize 5 tsize 10 (C5b) 9.16 -> 8.60 ms,
+// tsize 100 63.0 -> 61.6 ms, tsize 1000 (dim 4096) unchanged; dsize 1 tsize 10 (C5a) +0.6 %,
+// tsize 1000 (C5c) +1.5 %, so only many-plane cells (dsize >= 3, the 16-row-window regime) get it.
+// WF_SYN_PAD >= 0 forces the count (experiments).
+#ifndef WF_SYN_PAD
+#define WF_SYN_PAD -1
+#endif
+__host__ __device__ constexpr int syn_pad(int ds) { return WF_SYN_PAD >= 0 ? WF_SYN_PAD : (ds >= 3 ? 2 : 0); }
 template <int DS, int K, int WARPS, int TS>
-__global__ void __launch_bounds__((WARPS + 1) * 32)
+__global__ void __launch_bounds__((WARPS + 1 + syn_pad(DS)) * 32)
     syn_kernel(const SweepLaunch L, const PolSyn<DS> pol, const __grid_constant__ SynMaps maps) {
   using S = SynSmem<DS, K, WARPS>;
   extern __shared__ __align__(16) unsigned char syn_smem_raw[];
@@ -439,7 +450,7 @@ __global__ void __launch_bounds__((WARPS + 1) * 32)
     __syncthreads();
     if (warp == WARPS) {
       syn_feeder<DS, K, WARPS>(L, pol, sm, band, lane);
-    } else {
+    } else if (warp < WARPS) {
       SynWarp<DS, K, WARPS, TS> w(L, pol, maps, sm, band, warp, lane);
       w.run();
     }
@@ -478,14 +489,14 @@ cudaError_t launch_syn(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   }
   cudaError_t e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
-  kfn<<<L.grid, (W + 1) * 32, smem, s>>>(L, pol, maps);
+  kfn<<<L.grid, (W + 1 + syn_pad(DS)) * 32, smem, s>>>(L, pol, maps);
   return cudaGetLastError();
 }
 
 template <int DS, int K, int W>
 Variant make_syn() {
   using S = SynSmem<DS, K, W>;
-  return Variant{WF_FN_SYNTHETIC, DS, K, W, 1, (W + 1) * 32, S::bytes,
+  return Variant{WF_FN_SYNTHETIC, DS, K, W, 1, (W + 1 + syn_pad(DS)) * 32, S::bytes,
                  reinterpret_cast<const void*>(syn_kernel<DS, K, W, 0>), &launch_syn<DS, K, W>, 7};
 }
 
