@@ -98,7 +98,10 @@ typedef struct {
                            score lookup; codes outside the promise give unspecified scores */
   int32_t kernel;       /* kernel generation: 0 = the library's default for the function (tuned, DESIGN.md
                            §7); 4 = first generation (SEQCMP block hand-off v4, SYNTHETIC generic sweep);
-                           7 = second generation (SEQCMP per-row hand-off v7, SYNTHETIC wf_syn) */
+                           7 = second generation (SEQCMP per-row hand-off v7, SYNTHETIC wf_syn);
+                           8 = SYNTHETIC plane-split wf_syn (dsize 2..8, lane_cols = warps = skew = 1:
+                           one warp per float item on the same 32 columns); other combinations
+                           -> WF_EUNSUPPORTED */
   int32_t reserved[4];  /* must be zero */
 } wf_params;
 

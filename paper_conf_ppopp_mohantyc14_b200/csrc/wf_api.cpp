@@ -93,7 +93,12 @@ void defaults(const wf_params& p, int* k, int* w, int* d, int* impl) {
     // CTA with wf_syn for light cells; when a cell carries much FP work (dsize >= 3 with
     // tsize >= 1000, or dsize >= 5 with tsize >= 100) the generic sweep with 2 (dsize 3) or
     // 4 (dsize >= 5) warps per CTA wins (e.g. C5d 154 vs 197 ms).
-    const bool heavy = (p.dsize >= 3 && p.tsize >= 1000) || (p.dsize >= 5 && p.tsize >= 100);
+    // Exception, measured after the idle-warp padding of wf_syn (dsize >= 3): at dsize 5 with
+    // tsize >= 1000 the one-warp wf_syn CTA is faster again (C5d 154.5 -> 130.3 ms; dim 4096
+    // 38.5 -> 31.4 ms); at tsize 100 (32 vs 61 ms) and dsize 3 / 4 (116 / 131 vs 142 / 144 ms)
+    // the generic sweep stays ahead (tools/gpu_ps.sh).
+    const bool syn_pad_wins = p.dsize == 5 && p.tsize >= 1000;
+    const bool heavy = !syn_pad_wins && ((p.dsize >= 3 && p.tsize >= 1000) || (p.dsize >= 5 && p.tsize >= 100));
     *k = p.lane_cols ? p.lane_cols : 1;
     *w = p.warps ? p.warps : (heavy ? (p.dsize >= 5 ? 4 : 2) : 1);
     *d = p.skew ? p.skew : 1;
@@ -107,8 +112,8 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   const int cols = p->cols ? p->cols : p->dim;
   if (rows < 1 || rows > 65535) return fail(c, WF_EINVAL, "dim=%d out of range 1..65535", rows);
   if (cols < 1 || cols > 65535) return fail(c, WF_EINVAL, "cols=%d out of range 1..65535", cols);
-  if (p->kernel != 0 && p->kernel != 4 && p->kernel != 7)
-    return fail(c, WF_EINVAL, "kernel=%d must be 0 (default), 4 or 7", p->kernel);
+  if (p->kernel != 0 && p->kernel != 4 && p->kernel != 7 && p->kernel != 8)
+    return fail(c, WF_EINVAL, "kernel=%d must be 0 (default), 4, 7 or 8", p->kernel);
   for (int i = 0; i < 4; ++i)
     if (p->reserved[i]) return fail(c, WF_EINVAL, "reserved[%d] must be 0", i);
   if (p->alphabet < 0 || p->alphabet > 8) return fail(c, WF_EINVAL, "alphabet=%d out of range 0..8", p->alphabet);

@@ -254,10 +254,18 @@ const Variant* find(int fn, int dsize, int k, int warps, int skew, int impl) {
     for (size_t i = 0; i < n; ++i)
       if (t7[i].k == k && t7[i].warps == warps) return &t7[i];
   }
+  if (fn == WF_FN_SYNTHETIC && impl == 8) {   // plane-split wf_syn only; no fallback
+    const Variant* t7 = syn_table(&n);
+    for (size_t i = 0; i < n; ++i)
+      if (t7[i].impl == 8 && t7[i].dsize == dsize && t7[i].k == k && t7[i].warps == warps && t7[i].skew == skew)
+        return &t7[i];
+    return nullptr;
+  }
   if (fn == WF_FN_SYNTHETIC && skew == 1 && want_syn7(impl)) {
     const Variant* t7 = syn_table(&n);
     for (size_t i = 0; i < n; ++i)   // a wf_syn variant whose staging rings do not fit falls back to the generic sweep
-      if (t7[i].dsize == dsize && t7[i].k == k && t7[i].warps == warps && t7[i].smem <= 232448) return &t7[i];
+      if (t7[i].impl == 7 && t7[i].dsize == dsize && t7[i].k == k && t7[i].warps == warps && t7[i].smem <= 232448)
+        return &t7[i];
   }
   const Variant* t = table(&n);
   for (size_t i = 0; i < n; ++i)

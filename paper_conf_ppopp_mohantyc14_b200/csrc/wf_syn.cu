@@ -103,28 +103,44 @@ __device__ __forceinline__ void stg_gpu_u64_pred(bool p, unsigned long long* a, 
 #endif
 }
 
-template <int DS, int K, int WARPS, int TS>
+// PW >= 0: plane-split warp (impl 8, one column warp per band): the CTA runs DS compute warps
+// on the SAME 32 columns, warp PW computing float item d = PW (warp 0 also the two int fields).
+// The items of a cell are independent given (N, W, NW, u_i, v_j) (R5), so each warp's tsize
+// chain is one item deep instead of DS: the step is bound by one FMA chain's latency, not by
+// DS x tsize FFMA issues of one warp.
+template <int DS, int K, int WARPS, int TS, int PW = -1>
 struct SynWarp {
   using P = PolSyn<DS>;
   using S = SynSmem<DS, K, WARPS>;
   static constexpr int NF = S::NF, NWD = S::NWD, U = S::U, R = S::R, ROWB = S::ROWB;
   static constexpr int kOff = 30 % U;   // lane 31's rows of a block occupy contiguous staging slots
+  // does this warp compute / store / hand off field f
+  __host__ __device__ static constexpr bool use(int f) { return PW < 0 || (f < 2 ? PW == 0 : f - 2 == PW); }
+  static constexpr int kRd = PW < 0 ? 0 : PW;   // my consumed-rows counter: rprog[warp + kRd]
 
   // The synthetic cell of wf_cells.cuh::PolSyn (same single operations in the same order,
   // DESIGN.md R5/R11), with the tsize loop unrolled when tsize is a compile-time constant
   // (TS > 0; TS = 0: runtime trip count).
   __device__ __forceinline__ void cell(const uint32_t* N, const uint32_t* W, const uint32_t* NW, uint32_t ui,
                                        uint32_t vj, uint32_t* o) const {
-    o[0] = static_cast<uint32_t>(max(max(static_cast<int>(N[0]), static_cast<int>(NW[0])), static_cast<int>(W[0])) + 1);
-    o[1] = ((N[1] - NW[1]) + 1u) + W[1];
-    if constexpr (DS > 0) {
+    if (use(0)) {
+      o[0] = static_cast<uint32_t>(max(max(static_cast<int>(N[0]), static_cast<int>(NW[0])), static_cast<int>(W[0])) + 1);
+      o[1] = ((N[1] - NW[1]) + 1u) + W[1];
+    } else {
+      o[0] = 0u;
+      o[1] = 0u;
+    }
+    if constexpr (DS > 0 && (PW < 0 || PW < DS)) {
       const float THIRD = __uint_as_float(0x3EAAAAABu);
       const float A = __uint_as_float(0x3F7FF000u);
       const float SCALE = __uint_as_float(0x39800000u);
       const float c = __fmul_rn(__fmul_rn(__uint_as_float(ui), __uint_as_float(vj)), SCALE);
+      constexpr int D0 = PW < 0 ? 0 : PW, D1 = PW < 0 ? DS : PW + 1;   // my items [D0, D1)
       float x[DS];
 #pragma unroll
-      for (int d = 0; d < DS; ++d)
+      for (int d = 0; d < DS; ++d) x[d] = 0.f;
+#pragma unroll
+      for (int d = D0; d < D1; ++d)
         x[d] = __fmul_rn(__fadd_rn(__fadd_rn(__uint_as_float(N[2 + d]), __uint_as_float(NW[2 + d])),
                                    __uint_as_float(W[2 + d])),
                          THIRD);
@@ -132,14 +148,14 @@ struct SynWarp {
 #pragma unroll 100
         for (int t = 0; t < TS; ++t) {
 #pragma unroll
-          for (int d = 0; d < DS; ++d) x[d] = __fmaf_rn(x[d], A, c);
+          for (int d = D0; d < D1; ++d) x[d] = __fmaf_rn(x[d], A, c);
         }
       } else {
         const int ts = pol.tsize;
 #pragma unroll 4
         for (int t = 0; t < ts; ++t) {
 #pragma unroll
-          for (int d = 0; d < DS; ++d) x[d] = __fmaf_rn(x[d], A, c);
+          for (int d = D0; d < D1; ++d) x[d] = __fmaf_rn(x[d], A, c);
         }
       }
 #pragma unroll
@@ -181,6 +197,7 @@ struct SynWarp {
     const int slot = (row + kOff) & (R - 1);
 #pragma unroll
     for (int f = 0; f < NF; ++f) {
+      if (!use(f)) continue;
       uint32_t* dst = reinterpret_cast<uint32_t*>(stage_w + (size_t(f) * R + slot) * ROWB) + lane * K;
 #pragma unroll
       for (int m = 0; m < K; ++m) sts_u32_pred(p, dst + m, H[m][f]);
@@ -193,6 +210,7 @@ struct SynWarp {
     const int slot = (r + kOff) & (R - 1);
 #pragma unroll
     for (int f = 0; f < NF; ++f) {
+      if (!use(f)) continue;
       const uint32_t* src = reinterpret_cast<const uint32_t*>(stage_w + (size_t(f) * R + slot) * ROWB) + lane * K;
       uint32_t* dst = static_cast<uint32_t*>(L.out[f]) + int64_t(r - 1) * L.pitch + jrel;
 #pragma unroll
@@ -205,7 +223,7 @@ struct SynWarp {
   __device__ __forceinline__ void issue(int r, uint32_t (&w)[NWD]) const {
     const uint32_t* p = sm.slot(warp, r);
 #pragma unroll
-    for (int i = 0; i < NWD; ++i) w[i] = lds_vol_u32(p + i);
+    for (int i = 0; i < NWD; ++i) w[i] = (i == NF || use(i)) ? lds_vol_u32(p + i) : 0u;
   }
   // wait until a shared progress counter reaches `need` (seen caches the last value)
   __device__ __forceinline__ bool wait_ctr(const int* ctr, int need, int& seen) {
@@ -266,10 +284,11 @@ struct SynWarp {
         unsigned long long* g = gdst + size_t(row) * NF;
         (void)to_peer;
 #pragma unroll
-        for (int f = 0; f < NF; ++f) stg_sys_u64_pred(pub && glob, g + f, ll_pack(Np[K - 1][f], L.epoch));
+        for (int f = 0; f < NF; ++f)
+          if (use(f)) stg_sys_u64_pred(pub && glob, g + f, ll_pack(Np[K - 1][f], L.epoch));
       }
 #pragma unroll
-      for (int f = 0; f < NF; ++f) q[f] = __shfl_up_sync(0xffffffffu, Np[K - 1][f], 1);
+      for (int f = 0; f < NF; ++f) q[f] = use(f) ? __shfl_up_sync(0xffffffffu, Np[K - 1][f], 1) : 0u;
       qx = __shfl_up_sync(0xffffffffu, xr, 1);
     }
   }
@@ -306,7 +325,7 @@ struct SynWarp {
     for (int t0 = 0; t0 < T; t0 += UB) {
       // this block reads rows t0+2 .. t0+UB+1 of my ring (row t0+1 is already in pre)
       if (!wait_ctr(sm.wprog + warp, min(t0 + UB + 1, rows), seen_w)) return false;
-      if (lane == 0) sts_vol_i(sm.rprog + warp, t0 + 1);   // rows <= t0+1 of my ring consumed
+      if (lane == 0) sts_vol_i(sm.rprog + warp + kRd, t0 + 1);   // rows <= t0+1 of my ring consumed
       // lane 31 writes rows t0-30 .. t0-31+UB into the next ring: their slots must be free
       if (!last && !wait_ctr(sm.rprog + warp + 1, t0 - 31 + UB - kSynLL, seen_r)) return false;
       if (t0 % U == 0) {
@@ -339,7 +358,7 @@ struct SynWarp {
           if (lane == 0) {
 #pragma unroll
             for (int f = 0; f < NF; ++f)
-              tma_store_2d(&maps.m[f], stage_s + (f * R + ((r31_0 + kOff) & (R - 1))) * ROWB, wcol, r31_0 - 1);
+              if (use(f)) tma_store_2d(&maps.m[f], stage_s + (f * R + ((r31_0 + kOff) & (R - 1))) * ROWB, wcol, r31_0 - 1);
             bulk_commit();
           }
         } else {
@@ -349,7 +368,7 @@ struct SynWarp {
     }
     if (lane == 0) {
       bulk_wait_all();
-      sts_vol_i(sm.rprog + warp, rows + kSynLL + 64);
+      sts_vol_i(sm.rprog + warp + kRd, rows + kSynLL + 64);
     }
     if (L.trace && lane == 0) {
       L.trace[size_t(band) * kTraceSlots + 52 + warp] = globaltimer();
@@ -361,7 +380,7 @@ struct SynWarp {
 
 // Feeder warp: warp 0's west words (column-0 boundary planes, or the band's global LL ring
 // written by the previous band / slab) plus u_i, as row-tagged LL words in shared memory.
-template <int DS, int K, int WARPS>
+template <int DS, int K, int WARPS, int NPW = 1>
 __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS>& pol, const SynSmem<DS, K, WARPS>& sm,
                                            int band, int lane) {
   using S = SynSmem<DS, K, WARPS>;
@@ -376,6 +395,8 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
     const int need = feed + 31 - kSynLL;   // slot reuse: warp 0 has consumed those rows
     if (seen < need) {
       seen = lds_vol_i(sm.rprog + 0);
+#pragma unroll
+      for (int p = 1; p < NPW; ++p) seen = min(seen, lds_vol_i(sm.rprog + p));   // plane-split readers
       if (seen < need) {
         if (wd.expired(L)) return false;
         __nanosleep(64);
@@ -459,6 +480,39 @@ __global__ void __launch_bounds__((WARPS + 1 + syn_pad(DS)) * 32)
   }
 }
 
+// Plane-split kernel (impl 8): one 32-column band per CTA, DS compute warps (warp d computes
+// float item d, warp 0 also the int fields) + the feeder (warp DS), which recycles a west-ring
+// slot once every plane warp has consumed it.
+template <int DS, int TS, int PW>
+__device__ __forceinline__ void syn_ps_dispatch(const SweepLaunch& L, const PolSyn<DS>& pol, const SynMaps& maps,
+                                                const SynSmem<DS, 1, 1>& sm, int band, int warp, int lane) {
+  if constexpr (PW < DS) {
+    if (warp == PW) {
+      SynWarp<DS, 1, 1, TS, PW> w(L, pol, maps, sm, band, 0, lane);
+      w.run();
+    } else {
+      syn_ps_dispatch<DS, TS, PW + 1>(L, pol, maps, sm, band, warp, lane);
+    }
+  }
+}
+
+template <int DS, int TS>
+__global__ void __launch_bounds__((DS + 1) * 32)
+    syn_ps_kernel(const SweepLaunch L, const PolSyn<DS> pol, const __grid_constant__ SynMaps maps) {
+  using S = SynSmem<DS, 1, 1>;
+  extern __shared__ __align__(16) unsigned char syn_smem_raw[];
+  const S sm(syn_smem_raw);
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  for (int band = blockIdx.x; band < L.nbands; band += gridDim.x) {
+    if (threadIdx.x < 64) sm.rprog[threadIdx.x] = 0;   // rprog and wprog
+    __syncthreads();
+    if (warp == DS) syn_feeder<DS, 1, 1, DS>(L, pol, sm, band, lane);
+    else syn_ps_dispatch<DS, TS, 0>(L, pol, maps, sm, band, warp, lane);
+    __syncthreads();
+    if (run_failed(L)) return;
+  }
+}
+
 cudaError_t encode_plane_map_f(CUtensorMap* m, const SweepLaunch& L, int plane, int box_cols, int box_rows);
 
 namespace {
@@ -493,6 +547,40 @@ cudaError_t launch_syn(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   return cudaGetLastError();
 }
 
+template <int DS>
+cudaError_t launch_syn_ps(const SweepLaunch& L, cudaStream_t s, size_t smem) {
+  PolSyn<DS> pol{};
+  pol.u = static_cast<const float*>(L.row_in);
+  pol.v = static_cast<const float*>(L.col_in);
+  for (int d = 0; d < DS; ++d) {
+    pol.topf[d] = static_cast<const float*>(L.top[d]);
+    pol.leftf[d] = static_cast<const float*>(L.left[d]);
+  }
+  pol.tsize = L.tsize;
+  SynMaps maps;
+  memset(&maps, 0, sizeof maps);
+  for (int f = 0; f < 2 + DS; ++f) {
+    cudaError_t e = encode_plane_map_f(&maps.m[f], L, f, 32, syn_ut(DS));
+    if (e != cudaSuccess) return e;
+  }
+  auto kfn = syn_ps_kernel<DS, 0>;
+  if constexpr (DS == 5) {
+    if (L.tsize == 100) kfn = syn_ps_kernel<DS, 100>;
+    if (L.tsize == 1000) kfn = syn_ps_kernel<DS, 1000>;
+  }
+  cudaError_t e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  if (e != cudaSuccess) return e;
+  kfn<<<L.grid, (DS + 1) * 32, smem, s>>>(L, pol, maps);
+  return cudaGetLastError();
+}
+
+template <int DS>
+Variant make_syn_ps() {
+  using S = SynSmem<DS, 1, 1>;
+  return Variant{WF_FN_SYNTHETIC, DS, 1, 1, 1, (DS + 1) * 32, S::bytes,
+                 reinterpret_cast<const void*>(syn_ps_kernel<DS, 0>), &launch_syn_ps<DS>, 8};
+}
+
 template <int DS, int K, int W>
 Variant make_syn() {
   using S = SynSmem<DS, K, W>;
@@ -506,10 +594,12 @@ Variant make_syn() {
 
 const Variant* syn_table(size_t* n) {
 #ifdef WF_MIN_VARIANTS
-  static const Variant v[] = {WF_SYN7(1), WF_SYN7(5)};
+  static const Variant v[] = {WF_SYN7(1), WF_SYN7(5), make_syn_ps<5>()};
 #else
   static const Variant v[] = {WF_SYN7(0), WF_SYN7(1), WF_SYN7(2), WF_SYN7(3), WF_SYN7(4),
-                              WF_SYN7(5), WF_SYN7(6), WF_SYN7(7), WF_SYN7(8)};
+                              WF_SYN7(5), WF_SYN7(6), WF_SYN7(7), WF_SYN7(8),
+                              make_syn_ps<2>(), make_syn_ps<3>(), make_syn_ps<4>(), make_syn_ps<5>(),
+                              make_syn_ps<6>(), make_syn_ps<7>(), make_syn_ps<8>()};
 #endif
   *n = sizeof(v) / sizeof(v[0]);
   return v;

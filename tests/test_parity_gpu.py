@@ -300,6 +300,36 @@ def test_synthetic_variants(k, w, d):
     _check_syn(o, g)
 
 
+@pytest.mark.parametrize("dim", [1, 33, 257, 419])
+@pytest.mark.parametrize("tsize", [0, 7, 100])
+@pytest.mark.parametrize("dsize", [2, 3, 5, 8])
+def test_synthetic_plane_split(dim, tsize, dsize):
+    """kernel=8: one warp per float item on the same columns (R5: the items of a cell are
+    independent given its inputs) -- same grid as the oracle, bit-exact."""
+    o, g = _syn(dim, tsize, dsize, kernel=8, lane_cols=1, warps=1, skew=1)
+    _check_syn(o, g)
+
+
+@pytest.mark.parametrize("tsize", [100, 1000])
+def test_synthetic_plane_split_compiled_tsize(tsize):
+    o, g = _syn(300, tsize, 5, kernel=8, lane_cols=1, warps=1, skew=1)
+    _check_syn(o, g)
+
+
+@pytest.mark.parametrize("G", [2, 3])
+def test_synthetic_plane_split_slabs_and_rect(G):
+    o, g = _syn(333, 9, 5, kernel=8, lane_cols=1, warps=1, skew=1, ngpus=G)
+    _check_syn(o, g)
+    o, g = _syn(129, 9, 3, cols=300, kernel=8, lane_cols=1, warps=1, skew=1)
+    _check_syn(o, g)
+
+
+def test_synthetic_plane_split_rejects_single_item():
+    with pytest.raises(_abi.WfError) as ei:
+        _syn(64, 5, 1, kernel=8, lane_cols=1, warps=1, skew=1)
+    assert ei.value.status == _abi.WF_EUNSUPPORTED
+
+
 @pytest.mark.parametrize("G", [2, 3])
 def test_synthetic_local_slabs(G):
     o, g = _syn(333, 5, 2, ngpus=G)
@@ -318,12 +348,13 @@ def test_synthetic_c2_full_grid():
 
 
 @pytest.mark.slow
-@pytest.mark.parametrize("name,prefix", [("C5a", 64), ("C5b", 32), ("C5c", 8), ("C5d", 4)])
-def test_synthetic_c5_prefix_and_closed_forms(name, prefix):
+@pytest.mark.parametrize("name,prefix,kw", [("C5a", 64, {}), ("C5b", 32, {}), ("C5c", 8, {}), ("C5d", 4, {}),
+                                            ("C5d", 4, {"kernel": 8, "lane_cols": 1, "warps": 1, "skew": 1})])
+def test_synthetic_c5_prefix_and_closed_forms(name, prefix, kw):
     """C5 at full size: exact parity on a row prefix (a true prefix of the grid), plus the
     closed forms i0 = (i-1)+(j-1), i1 = i*j and the value range on EVERY cell."""
     c = workloads.CONFIGS[name]
-    o, g = _syn(c.dim, c.tsize, c.dsize, m_compute=prefix)
+    o, g = _syn(c.dim, c.tsize, c.dsize, m_compute=prefix, **kw)
     _check_syn(o, g, rows=prefix)
     i = np.arange(1, c.dim + 1, dtype=np.int64)[:, None]
     j = np.arange(1, c.dim + 1, dtype=np.int64)[None, :]

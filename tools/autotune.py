@@ -39,10 +39,11 @@ import workloads  # noqa: E402
 from paper_conf_ppopp_mohantyc14_b200.wf import Wavefront  # noqa: E402
 
 # impl = wf_params.kernel: 4 = first generation (NW v4 / generic synthetic sweep),
-# 7 = second generation (NW v7 / wf_syn); Nash has one kernel (0)
+# 7 = second generation (NW v7 / wf_syn), 8 = plane-split wf_syn (synthetic, dsize >= 2, k = w = d = 1);
+# Nash has one kernel (0)
 SEARCH = {
     "seqcmp": {"k": [2, 4, 8], "w": [1, 2, 4], "d": [1, 2], "impl": [4, 7]},
-    "synthetic": {"k": [1, 2], "w": [1, 2, 4], "d": [1, 2], "impl": [7, 4]},
+    "synthetic": {"k": [1, 2], "w": [1, 2, 4], "d": [1, 2], "impl": [7, 4, 8]},
     "nash": {"k": [1], "w": [1, 2, 4, 8], "d": [1], "impl": [0]},
 }
 

@@ -47,8 +47,11 @@ def main():
     for dim in a.dim:
         ins = inputs(a.fn, dim, a.dsize, dev, a.cols)
         for v in a.variants:
-            k, w, d = (int(s) for s in v.split(","))
+            parts = [int(s) for s in v.split(",")]   # k,w,d[,kernel]
+            k, w, d = parts[:3]
             kw = dict(lane_cols=k, warps=w, skew=d)
+            if len(parts) > 3:
+                kw.update(kernel=parts[3])
             if a.fn == "seqcmp":
                 kw.update(alphabet=a.alphabet)
             if a.fn == "synthetic":

@@ -38,7 +38,8 @@ def default_choice(fn, dim, tsize, dsize):
         return (4, 2, 1, 4)
     if fn == "nash":
         return (1, 2, 1, 0)
-    heavy = (dsize >= 3 and tsize >= 1000) or (dsize >= 5 and tsize >= 100)
+    syn_pad_wins = dsize == 5 and tsize >= 1000
+    heavy = not syn_pad_wins and ((dsize >= 3 and tsize >= 1000) or (dsize >= 5 and tsize >= 100))
     return (1, 4 if dsize >= 5 else 2, 1, 4) if heavy else (1, 1, 1, 7)
 
 
