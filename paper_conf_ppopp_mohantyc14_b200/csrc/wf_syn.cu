@@ -36,8 +36,15 @@ constexpr int kSynLL = 128;   // rows per shared west LL ring (power of 2)
 //    (large tsize) a step is expensive and small blocks win, with light cells the per-block
 //    cost dominates: UB = 16 / 8 / 4 for tsize x dsize < 40 / < 1000 (or runtime) / >= 1000.
 __host__ __device__ constexpr int syn_ut(int ds) { return ds <= 2 ? 32 : 16; }
+#ifndef WF_SYN_UB_LIGHT
+#define WF_SYN_UB_LIGHT 16   // experiments: hand-off block of light cells (tsize x dsize < 40)
+#endif
+#ifndef WF_SYN_UB_MID
+#define WF_SYN_UB_MID 8      // experiments: hand-off block of medium cells (< 1000, or runtime tsize)
+#endif
 __host__ __device__ constexpr int syn_ub(int ts, int ds) {
-  return ts == 0 ? 8 : (ts * (ds > 0 ? ds : 1) >= 1000 ? 4 : ts * (ds > 0 ? ds : 1) >= 40 ? 8 : 16);
+  return ts == 0 ? WF_SYN_UB_MID
+                 : (ts * (ds > 0 ? ds : 1) >= 1000 ? 4 : ts * (ds > 0 ? ds : 1) >= 40 ? WF_SYN_UB_MID : WF_SYN_UB_LIGHT);
 }
 
 struct SynMaps {
