@@ -387,6 +387,15 @@ struct SynWarp {
 
 // Feeder warp: warp 0's west words (column-0 boundary planes, or the band's global LL ring
 // written by the previous band / slab) plus u_i, as row-tagged LL words in shared memory.
+// Feeder back-off between LL polls: spin for few planes (C5a 4.114 -> 4.075 ms, C2 -0.4 %),
+// 64 ns for many planes (C5b +0.2 % when spinning); profiles/r01_syn_feed_ab.txt.
+// WF_SYN_FEED_NS >= 0 forces it (experiments).
+#ifndef WF_SYN_FEED_NS
+#define WF_SYN_FEED_NS -1
+#endif
+__host__ __device__ constexpr unsigned syn_feed_ns(int ds) {
+  return WF_SYN_FEED_NS >= 0 ? unsigned(WF_SYN_FEED_NS) : (ds <= 2 ? 0u : 64u);
+}
 template <int DS, int K, int WARPS, int NPW = 1>
 __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS>& pol, const SynSmem<DS, K, WARPS>& sm,
                                            int band, int lane) {
@@ -446,10 +455,10 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
         __syncwarp();
         if (lane == 0) st_relaxed_sys_u32(L.ack_prev, L.epoch);   // predecessor slab may reuse this ring
       }
-      if (n < 32) __nanosleep(64);
+      if (syn_feed_ns(DS) && n < 32) __nanosleep(syn_feed_ns(DS));
     } else {
       if (wd.expired(L)) return false;
-      __nanosleep(64);
+      if (syn_feed_ns(DS)) __nanosleep(syn_feed_ns(DS));
     }
   }
   return true;
