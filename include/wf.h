@@ -97,10 +97,11 @@ typedef struct {
                            row_in/col_in is < alphabet (e.g. 4 for DNA) -- enables the byte-permute
                            score lookup; codes outside the promise give unspecified scores */
   int32_t kernel;       /* kernel generation: 0 = the library's default for the function (tuned, DESIGN.md
-                           §7); 4 = first generation (SEQCMP block hand-off v4, SYNTHETIC generic sweep);
-                           7 = second generation (SEQCMP per-row hand-off v7, SYNTHETIC wf_syn);
-                           8 = SYNTHETIC plane-split wf_syn (dsize 2..8, lane_cols = warps = skew = 1:
-                           one warp per float item on the same 32 columns); other combinations
+                           §7).  SEQCMP: 8 = the lockstep lane pipeline (wf_nw8.cu; the default where its
+                           (lane_cols, warps) is compiled, skew 1), 4 = the block hand-off sweep (wf_nw.cuh;
+                           every other tuning).  SYNTHETIC: 4 = the generic sweep, 7 = wf_syn (the default
+                           at skew 1), 8 = plane-split wf_syn (dsize 2..8, lane_cols = warps = skew = 1:
+                           one warp per float item on the same 32 columns).  Other combinations
                            -> WF_EUNSUPPORTED */
   int32_t reserved[4];  /* must be zero */
 } wf_params;

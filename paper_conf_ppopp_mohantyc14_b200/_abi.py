@@ -8,7 +8,7 @@ import ctypes
 import os
 
 HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.environ.get("WF_LIB_OVERRIDE") or os.path.join(HERE, "libwf.so")   # override: perf experiments
+LIB_PATH = os.path.join(HERE, "libwf.so")
 
 WF_MAX_PLANES = 10
 WF_IPC_HANDLE_BYTES = 64

@@ -78,8 +78,11 @@ struct Plan {
 void defaults(const wf_params& p, int* k, int* w, int* d, int* impl) {
   *impl = p.kernel;
   if (p.fn == WF_FN_SEQCMP) {
-    *k = p.lane_cols ? p.lane_cols : 4;
-    *w = p.warps ? p.warps : 2;
+    // generation 8 (wf_nw8.cu): 4 compute warps of K = 2 columns per lane, one long lane
+    // pipeline with per-row hand-offs; generation 4 keeps (4, 2)
+    const bool g4 = p.kernel == 4;
+    *k = p.lane_cols ? p.lane_cols : (g4 ? 4 : 2);
+    *w = p.warps ? p.warps : (g4 ? 2 : 4);
     *d = p.skew ? p.skew : 1;
   } else if (p.fn == WF_FN_NASH) {
     // one warp per column: lane_cols and skew are fixed at 1; 2 columns per CTA measured
@@ -114,6 +117,8 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   if (cols < 1 || cols > 65535) return fail(c, WF_EINVAL, "cols=%d out of range 1..65535", cols);
   if (p->kernel != 0 && p->kernel != 4 && p->kernel != 7 && p->kernel != 8)
     return fail(c, WF_EINVAL, "kernel=%d must be 0 (default), 4, 7 or 8", p->kernel);
+  if (p->fn == WF_FN_SEQCMP && p->kernel == 7)
+    return fail(c, WF_EUNSUPPORTED, "kernel=7: SEQCMP has generations 4 and 8 (the per-row v7 kernel was retired, DESIGN.md §12)");
   for (int i = 0; i < 4; ++i)
     if (p->reserved[i]) return fail(c, WF_EINVAL, "reserved[%d] must be 0", i);
   if (p->alphabet < 0 || p->alphabet > 8) return fail(c, WF_EINVAL, "alphabet=%d out of range 0..8", p->alphabet);
@@ -317,9 +322,14 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   if (p->max_ctas && (int)p->max_ctas < c->grid) c->grid = (int)p->max_ctas;
   if (c->grid < 1) c->grid = 1;
 
-  c->edge_bytes = (size_t)pl.nbands * wfk::edge_stride(p->dim) * pl.nf * sizeof(unsigned long long);
+  // per band: the inbound LL ring (edge_stride rows) plus 32 slots of slack on each side (the
+  // generation-8 ring is addressed at +32 so that ramp-up / drain rows never leave it)
+  c->edge_bytes = (size_t)pl.nbands * (wfk::edge_stride(p->dim) + 64) * pl.nf * sizeof(unsigned long long);
   e = cudaMalloc(&c->base, kCtrlBytes + c->edge_bytes);
-  if (e == cudaSuccess) e = cudaMemset(c->base, 0, kCtrlBytes + c->edge_bytes);
+  // control block 0; edge rings 0x80 bytes: the generation-8 EMPTY word (0x80808080), and a tag
+  // no epoch ever takes for the LL-word generations
+  if (e == cudaSuccess) e = cudaMemset(c->base, 0, kCtrlBytes);
+  if (e == cudaSuccess) e = cudaMemset(static_cast<char*>(c->base) + kCtrlBytes, 0x80, c->edge_bytes);
   if (e == cudaSuccess) {
     c->ack = static_cast<unsigned*>(c->base);
     c->edge = reinterpret_cast<unsigned long long*>(static_cast<char*>(c->base) + kCtrlBytes);

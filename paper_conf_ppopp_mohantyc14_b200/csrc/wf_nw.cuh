@@ -356,25 +356,17 @@ struct NwWarp {
     int32_t Win = (lane == 0) ? w00 : q[0];
     uint32_t Xin = (lane == 0) ? x00 : xq[0];
 #pragma unroll
-#ifndef WF_NW_ABL
-#define WF_NW_ABL 0   // performance archaeology only (wrong grids): 1 no STS, 2 no x shuffles, 4 no w0 shuffle
-#endif
     for (int u = 0; u < U; ++u) {
       const int row = t0 + u - lane + 1;
-      const int32_t w0n = (WF_NW_ABL & 4) ? u : __shfl_sync(0xffffffffu, wv, (u + 1) & (U - 1));   // next row of lane 0
-      const uint32_t x0n = (WF_NW_ABL & 2) ? 1u : __shfl_sync(0xffffffffu, xv, (u + 1) & (U - 1));
+      const int32_t w0n = __shfl_sync(0xffffffffu, wv, (u + 1) & (U - 1));   // next row of lane 0
+      const uint32_t x0n = __shfl_sync(0xffffffffu, xv, (u + 1) & (U - 1));
       int32_t H[K];
       int32_t Pl;
       cells_p(Win, Xin, H, Pl);
       const int32_t PL = (lane == 31) ? w0n : Pl;
       const int32_t src = __viaddmax_s32(Win, gL, PL);
       const uint32_t xsrc = (lane == 31) ? x0n : Xin;
-      if constexpr ((WF_NW_ABL & 1) != 0) {
-        prevW = Win;
-#pragma unroll
-        for (int m = 0; m < K; ++m) Np[m] = H[m];
-        if (u == U - 1) stage_store(row, H);
-      } else if constexpr (EDGE) {
+      if constexpr (EDGE) {
         const bool active = row >= 1 && row <= rows;
         prevW = active ? Win : prevW;
 #pragma unroll
@@ -387,7 +379,7 @@ struct NwWarp {
         stage_store(row, H);
       }
       Win = __shfl_sync(0xffffffffu, src, src_lane);
-      if constexpr ((WF_NW_ABL & 2) == 0) Xin = __shfl_sync(0xffffffffu, xsrc, src_lane);
+      Xin = __shfl_sync(0xffffffffu, xsrc, src_lane);
     }
     // lanes 1..31 carry their next west input into the next block in q[0]
     q[0] = Win;

@@ -16,8 +16,7 @@
 namespace wfk {
 
 cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols, int box_rows);
-cudaError_t launch_nw_kernel(void (*kfn)(const SweepLaunch, const PolSeq, const CUtensorMap),
-                             void (*kcl)(const SweepLaunch, const PolSeq, const CUtensorMap), const SweepLaunch& L,
+cudaError_t launch_nw_kernel(void (*kfn)(const SweepLaunch, const PolSeq, const CUtensorMap), const SweepLaunch& L,
                              const PolSeq& pol, const CUtensorMap& tmap, int threads, size_t smem, cudaStream_t s);
 
 // One CTA: value max, then the smallest row among the lanes holding it, then the smallest
@@ -84,7 +83,7 @@ cudaError_t launch_sw(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   auto kfn = (L.alphabet >= 1 && L.alphabet <= 8) ? nw_kernel<K, W, D, U, true, true> : nw_kernel<K, W, D, U, false, true>;
   e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
-  return launch_nw_kernel(kfn, nullptr, L, pol, tmap, (W + 2) * 32, smem, s);
+  return launch_nw_kernel(kfn, L, pol, tmap, (W + 2) * 32, smem, s);
 }
 
 template <int K, int W, int D>

@@ -87,48 +87,9 @@ namespace {
 
 }  // namespace
 
-// Launch an NW-family kernel.  With a cluster kernel `kcl` and WF_NW_CLUSTER=<size> (2, 4 or 8)
-// the grid is launched as clusters of that many CTAs (band-to-band hand-off through
-// distributed shared memory, wf_nw.cuh) when a whole number of co-resident clusters covers
-// the grid; otherwise as a plain persistent grid (the default: measured faster).
-cudaError_t launch_nw_kernel(void (*kfn)(const SweepLaunch, const PolSeq, const CUtensorMap),
-                             void (*kcl)(const SweepLaunch, const PolSeq, const CUtensorMap), const SweepLaunch& L,
+// Launch an NW-family kernel of generation 4 as a plain persistent grid.
+cudaError_t launch_nw_kernel(void (*kfn)(const SweepLaunch, const PolSeq, const CUtensorMap), const SweepLaunch& L,
                              const PolSeq& pol, const CUtensorMap& tmap, int threads, size_t smem, cudaStream_t s) {
-  const char* env = getenv("WF_NW_CLUSTER");
-  const int cs = env ? atoi(env) : 0;
-  if (kcl && (cs == 2 || cs == 4 || cs == 8) && L.nbands >= 2 * cs && L.grid >= 2 * cs) {
-    cudaError_t e = cudaFuncSetAttribute(kcl, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-    if (e != cudaSuccess) return e;
-    cudaLaunchConfig_t cfg = {};
-    cudaLaunchAttribute at[1];
-    at[0].id = cudaLaunchAttributeClusterDimension;
-    at[0].val.clusterDim.x = cs;
-    at[0].val.clusterDim.y = 1;
-    at[0].val.clusterDim.z = 1;
-    cfg.blockDim = dim3(threads);
-    cfg.dynamicSmemBytes = smem;
-    cfg.stream = s;
-    cfg.attrs = at;
-    cfg.numAttrs = 1;
-    int g = (L.grid / cs) * cs;
-    cfg.gridDim = dim3(g);
-    int ncl = 0;
-    if (cudaOccupancyMaxActiveClusters(&ncl, reinterpret_cast<const void*>(kcl), &cfg) != cudaSuccess) {
-      cudaGetLastError();
-      ncl = 0;
-    }
-    if (getenv("WF_NW_CLUSTER_DEBUG")) fprintf(stderr, "wf: cluster %d launch grid %d, max active clusters %d\n", cs, g, ncl);
-    g = g < ncl * cs ? g : ncl * cs;
-    if (g >= 2 * cs) {
-      SweepLaunch Lc = L;
-      Lc.grid = g;
-      Lc.cluster = cs;
-      cfg.gridDim = dim3(g);
-      e = cudaLaunchKernelEx(&cfg, kcl, Lc, pol, tmap);
-      if (e == cudaSuccess) return cudaGetLastError();
-      cudaGetLastError();
-    }
-  }
   SweepLaunch Lp = L;
   Lp.cluster = 0;
   kfn<<<L.grid, threads, smem, s>>>(Lp, pol, tmap);
@@ -154,11 +115,7 @@ cudaError_t launch_nw(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   auto kfn = (L.alphabet >= 1 && L.alphabet <= 8) ? nw_kernel<K, W, D, U, true> : nw_kernel<K, W, D, U, false>;
   e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
-  decltype(kfn) kcl = nullptr;
-  if constexpr (K == 4 && W == 2 && D == 1)   // the default C4 variant also exists as a cluster kernel
-    kcl = (L.alphabet >= 1 && L.alphabet <= 8) ? nw_kernel<K, W, D, U, true, false, true>
-                                               : nw_kernel<K, W, D, U, false, false, true>;
-  return launch_nw_kernel(kfn, kcl, L, pol, tmap, (W + 2) * 32, smem, s);   // + I/O warp + x-staging warp
+  return launch_nw_kernel(kfn, L, pol, tmap, (W + 2) * 32, smem, s);   // + I/O warp + x-staging warp
 }
 
 template <int K, int W, int D>
@@ -225,34 +182,21 @@ const Variant* table(size_t* n) {
   return v;
 }
 
-// Kernel generation (wf_params.kernel; the WF_NW_IMPL / WF_SYN_IMPL environment variables
-// override it for experiments).  SEQCMP at skew 1: v4 (block hand-offs) unless 7 is asked --
-// v4 measured faster on C4.
-bool want_nw7(int impl) {
-  const char* e = getenv("WF_NW_IMPL");
-  if (e && e[0]) return e[0] == '7';
-  return impl == 7;
-}
-
-// SYNTHETIC at skew 1 runs the wf_syn.cu kernel unless generation 4 (the generic sweep) is asked
-bool want_syn7(int impl) {
-  const char* e = getenv("WF_SYN_IMPL");
-  if (e && e[0]) return e[0] != '4';
-  return impl != 4;
-}
-
 const Variant* find(int fn, int dsize, int k, int warps, int skew, int impl) {
   size_t n;
+  // SEQCMP: generation 8 (the default, wf_nw8.cu) for its compiled (K, warps) at skew 1; every
+  // other tuning -- or kernel = 4 -- runs generation 4 (wf_nw.cuh, wf_sw.cu)
+  if (fn == WF_FN_SEQCMP && skew == 1 && (impl == 0 || impl == 8)) {
+    const Variant* t8 = nw8_table(&n);
+    for (size_t i = 0; i < n; ++i)
+      if (t8[i].dsize == dsize && t8[i].k == k && t8[i].warps == warps) return &t8[i];
+    if (impl == 8) return nullptr;
+  }
   if (fn == WF_FN_SEQCMP && dsize == 1) {   // local alignment (Smith-Waterman)
     const Variant* ts = sw_table(&n);
     for (size_t i = 0; i < n; ++i)
       if (ts[i].k == k && ts[i].warps == warps && ts[i].skew == skew) return &ts[i];
     return nullptr;
-  }
-  if (fn == WF_FN_SEQCMP && skew == 1 && want_nw7(impl)) {
-    const Variant* t7 = nw7_table(&n);
-    for (size_t i = 0; i < n; ++i)
-      if (t7[i].k == k && t7[i].warps == warps) return &t7[i];
   }
   if (fn == WF_FN_SYNTHETIC && impl == 8) {   // plane-split wf_syn only; no fallback
     const Variant* t7 = syn_table(&n);
@@ -261,7 +205,7 @@ const Variant* find(int fn, int dsize, int k, int warps, int skew, int impl) {
         return &t7[i];
     return nullptr;
   }
-  if (fn == WF_FN_SYNTHETIC && skew == 1 && want_syn7(impl)) {
+  if (fn == WF_FN_SYNTHETIC && skew == 1 && impl != 4) {   // wf_syn unless generation 4 (the generic sweep) is asked
     const Variant* t7 = syn_table(&n);
     for (size_t i = 0; i < n; ++i)   // a wf_syn variant whose staging rings do not fit falls back to the generic sweep
       if (t7[i].impl == 7 && t7[i].dsize == dsize && t7[i].k == k && t7[i].warps == warps && t7[i].smem <= 232448)

@@ -16,8 +16,8 @@ struct Variant {
   int impl;            // kernel generation (SEQCMP: 4 = block hand-offs, 7 = per-row hand-offs)
 };
 
-// SEQCMP v7 variants (wf_nw7.cu)
-const Variant* nw7_table(size_t* n);
+// SEQCMP v8 variants (wf_nw8.cu): global (dsize 0) and local / Smith-Waterman (dsize 1)
+const Variant* nw8_table(size_t* n);
 // SEQCMP local (Smith-Waterman) variants (wf_sw.cu); looked up with dsize = 1
 const Variant* sw_table(size_t* n);
 // SYNTHETIC v7 variants (wf_syn.cu)

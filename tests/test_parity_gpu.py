@@ -55,22 +55,30 @@ def test_seqcmp_variants(k, w, d, dim, alphabet):
     assert np.array_equal(H, g)
 
 
-@pytest.mark.parametrize("form", ["0", "1"])
-@pytest.mark.parametrize("k,w", [(4, 1), (4, 2), (2, 2), (2, 4), (8, 1)])
-@pytest.mark.parametrize("dim", [1, 33, 64, 97, 777, 1100])
-@pytest.mark.parametrize("alphabet", [0, 4])
-def test_seqcmp_v7_kernel(monkeypatch, form, k, w, dim, alphabet):
-    """The per-row hand-off kernel (wf_nw7.cu, opt-in via WF_NW_IMPL=7) against the oracle."""
-    monkeypatch.setenv("WF_NW_IMPL", "7")
-    monkeypatch.setenv("WF_NW7_FORM", form)
-    H, g = _seq(dim, lane_cols=k, warps=w, skew=1, seed=(dim + 5, dim + 6), alphabet=alphabet)
+NW8_VARIANTS = [(2, 4), (2, 2), (1, 4), (1, 8), (4, 2), (4, 1), (2, 1)]
+
+
+@pytest.mark.parametrize("k,w", NW8_VARIANTS)
+@pytest.mark.parametrize("dim", [1, 33, 64, 97, 777, 1100, 3001])
+def test_seqcmp_generation8_variants(k, w, dim):
+    """Every compiled (lane_cols, warps) of the lockstep lane pipeline (wf_nw8.cu, kernel=8):
+    one band, several bands, ragged last band, a ring lap (rows > 64) and ramp / drain blocks."""
+    H, g = _seq(dim, lane_cols=k, warps=w, skew=1, kernel=8, seed=(dim + 5, dim + 6))
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.parametrize("k,w,d", [(4, 2, 1), (2, 4, 1), (4, 1, 2)])
+@pytest.mark.parametrize("dim", [33, 777, 1100])
+def test_seqcmp_generation4_kernel(k, w, d, dim):
+    """The block hand-off generation (wf_nw.cuh, kernel=4) stays correct as the comparison kernel."""
+    H, g = _seq(dim, lane_cols=k, warps=w, skew=d, kernel=4, seed=(dim + 7, dim + 8), alphabet=4)
     assert np.array_equal(H, g)
 
 
 @pytest.mark.parametrize("G", [2, 3])
-def test_seqcmp_v7_local_slabs(monkeypatch, G):
-    monkeypatch.setenv("WF_NW_IMPL", "7")
-    H, g = _seq(1000, lane_cols=4, warps=2, skew=1, ngpus=G, alphabet=4)
+@pytest.mark.parametrize("kernel", [4, 8])
+def test_seqcmp_generations_local_slabs(G, kernel):
+    H, g = _seq(1000, ngpus=G, kernel=kernel, alphabet=4)
     assert np.array_equal(H, g)
 
 
