@@ -60,6 +60,9 @@ namespace nw8 {
 #ifndef WF_NW8_U
 #define WF_NW8_U 16    // steps per lockstep block (A/B: 8 and 4 slower, profiles/r02_nw8_ab.txt)
 #endif
+#ifndef WF_NW8_DPRE
+#define WF_NW8_DPRE 1  // blocks ahead the helper loads the inbound words (A/B 1 / 2 / 3: 1.96 / 2.02 / 2.06 ms)
+#endif
 
 constexpr int RR = 64;         // slots per shared ring (power of 2, > 2U)
 constexpr int SR = 128;        // staging rows per warp (power of 2, = 4 TMA boxes)
@@ -403,8 +406,8 @@ __device__ __noinline__ Slow4 slow_quad(const SweepLaunch& L, const int32_t* g, 
 // The helper warp (warp WARPS): all global-memory hand-off traffic of the band.  It runs the
 // CTA's block clock (one barrier per block) and, in CTA block j,
 //   inbound  (band > 0 or slab > 0): writes the west words of warp 0's block j+1 -- rows
-//            (j+1)U+2 .. (j+2)U+1, loaded during block j-1 -- into shared ring 0 after checking
-//            them, resets their global slots, and loads the words of block j+2;
+//            (j+1)U+2 .. (j+2)U+1, loaded DPRE blocks earlier -- into shared ring 0 after checking
+//            them, resets their global slots, and loads the words of block j+1+DPRE;
 //   outbound (a next band / slab exists): forwards the east words the last compute warp stored
 //            into ring WARPS during block j-1 to the next band's / slab's global ring.
 // Lane q < U/4 handles quad q (rows r0+4q .. r0+4q+3) of a block.
@@ -423,7 +426,8 @@ struct Helper {
   int32_t* gin;
   int32_t* gout;
   int4 emptyq;
-  int4 pre;           // inbound quad loaded one block ahead
+  static constexpr int DP = WF_NW8_DPRE;
+  int4 pre[DP];       // inbound quads of the next DP blocks (pre[0] = the next to deliver)
   bool failed = false;
   Watchdog wd;
 
@@ -442,27 +446,33 @@ struct Helper {
     outbound = gout != nullptr;
     const int32_t e = lds32(saddr(sm.ctl + 31));   // EMPTY, written by the kernel prologue (opaque to ptxas)
     emptyq = make_int4(e, e, e, e);
-    pre = make_int4(0, 0, 0, 0);
+#pragma unroll
+    for (int i = 0; i < DP; ++i) pre[i] = make_int4(0, 0, 0, 0);
   }
 
   // inbound quad of lane q for the block of warp 0 starting at local step s0 (rows s0+2+4q ..)
   __device__ __forceinline__ int rq(int s0) const { return s0 + 2 + 4 * lane; }
-  __device__ __forceinline__ void load_pre(int s0) {
+  __device__ __forceinline__ int4 load_quad(int s0) const {
     const int r = rq(s0);
-    pre = (mine && r <= rows) ? ldg128_sys(gin + r) : emptyq;
+    return (mine && r <= rows) ? ldg128_sys(gin + r) : emptyq;
   }
-  // check the preloaded quad of block s0, spin if stale, store it into ring 0, reset its slots
+  // check the quad of block s0 loaded DP blocks ago (pre[0]), spin if stale, store it into ring 0,
+  // reset its global slots; then shift the queue and load block s0 + DP U
   __device__ __forceinline__ void deliver(int s0) {
     const int r = rq(s0);
     const bool need = mine && r <= rows;
-    const bool st = need && quad_stale(pre, r, rows);
+    int4 v = pre[0];
+    const bool st = need && quad_stale(v, r, rows);
     if (!failed && __any_sync(FULL, st)) {
       const Slow4 w = slow_quad(L, gin + r, r, rows, need);
       failed = w.failed != 0;
-      if (need) pre = w.v;
+      if (need) v = w.v;
     }
-    if (mine) sts128(ring0 + slot(r), pre);
+    if (mine) sts128(ring0 + slot(r), v);
     if (need) stg128_sys(gin + r, emptyq);   // consumed: reset for the next run
+#pragma unroll
+    for (int i = 0; i + 1 < DP; ++i) pre[i] = pre[i + 1];
+    pre[DP - 1] = load_quad(s0 + DP * U);
   }
   // forward the east words the last compute warp stored during its block s0 (rows s0-30 ..)
   __device__ __forceinline__ void forward(int s0) {
@@ -510,17 +520,14 @@ struct Helper {
           __nanosleep(32);
         }
       }
-      load_pre(0);
+#pragma unroll
+      for (int i = 0; i < DP; ++i) pre[i] = load_quad(i * U);
       deliver(0);
-      load_pre(U);
     }
     cta_bar<NT>();   // warp 0's first block reads what the prologue stored
     for (int B = 0; B < Tc; B += U) {
       // B = CTA step of this block's start; warp 0's current block has local start s0 = B
-      if (inbound && B + U < Tw) {   // warp 0's next block starts at local step B + U
-        deliver(B + U);
-        load_pre(B + 2 * U);
-      }
+      if (inbound && B + U < Tw) deliver(B + U);   // warp 0's next block starts at local step B + U
       if (outbound && B >= U) {       // the last warp's block that ended at this block's start
         const int s0 = B - U - Ll;
         if (s0 >= 0 && s0 < Tw) forward(s0);
