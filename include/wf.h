@@ -92,7 +92,9 @@ typedef struct {
   uint32_t transport;   /* wf_transport for ngpus > 1: only WF_TRANSPORT_P2P is built; NCCL ->
                            WF_EUNSUPPORTED */
   uint32_t max_ctas;    /* 0 = all resident CTAs; else an upper bound (tests of the band loop) */
-  uint64_t watchdog_cycles; /* spin budget per dependency wait (SM clock cycles); 0 = default 2^32 */
+  uint64_t watchdog_cycles; /* spin budget per dependency wait (SM clock cycles); 0 = default: the larger of
+                               2^32 and 4x the expected pipeline fill (bands x slabs x 64 rows x the
+                               per-step cell cost estimate of fn / tsize / dsize) */
   int32_t alphabet;     /* SEQCMP: 0 = residue codes may be any byte value; 1..8 = every code in
                            row_in/col_in is < alphabet (e.g. 4 for DNA) -- enables the byte-permute
                            score lookup; codes outside the promise give unspecified scores */
@@ -181,14 +183,20 @@ wf_status wf_destroy(struct wf_ctx* c);
 const char* wf_last_error(const struct wf_ctx* c);
 
 /* Single-process multi-slab: make `next` (slab g+1) the consumer of `prev` (slab g).
- * Enables peer access when the devices differ (WF_ECOMM if impossible). */
+ * Enables peer access when the devices differ (WF_ECOMM if impossible).  WF_EINVAL unless the two
+ * contexts describe the same problem and tuning with prev's last column adjacent to next's first;
+ * WF_ESTATE if either context has already run (linked slabs pair their runs by epoch: link first,
+ * then issue the same sequence of wf_run calls on every slab). */
 wf_status wf_link_local(struct wf_ctx* prev, struct wf_ctx* next);
 
 /* One process per GPU: export this context's exchange buffer (control word + inbound edge
  * ring, one cudaMalloc) as a CUDA IPC handle (WF_IPC_HANDLE_BYTES bytes written to `handle`). */
 wf_status wf_ipc_handle(struct wf_ctx* c, void* handle);
 
-/* One process per GPU: open the neighbours' exchange buffers from their handle bytes.
+/* One process per GPU: open the neighbours' exchange buffers from their handle bytes; must be
+ * called before the context's first wf_run (WF_ESTATE otherwise), and every rank then issues
+ * the same sequence of wf_run calls (a rank that runs more often than its neighbour waits for
+ * words that never come and reports WF_ETIMEOUT).
  * prev_handle: rank-1's handle (NULL on rank 0) -- this slab acknowledges each drained run
  * into it.  next_handle: rank+1's handle (NULL on the last rank) -- this slab's east edge is
  * stored into its ring over NVLink.  WF_EINVAL if a required handle is missing, WF_ECOMM if

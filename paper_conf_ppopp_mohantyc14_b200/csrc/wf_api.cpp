@@ -38,11 +38,15 @@ struct wf_ctx {
   unsigned long long* next_edge = nullptr; // next slab's band-0 ring (peer / IPC / local)
   void* next_ipc_base = nullptr;
   int* err = nullptr;                      // device error word
+  int* err_host = nullptr;                 // pinned copy of the error word after each run (async D2H)
+  uint64_t watchdog = 0;                   // effective per-wait budget (SM cycles)
+  uint32_t reported = 0;                   // epoch whose device error was already returned
   unsigned long long* trace = nullptr;     // WF_TRACE=1 timeline buffer (diagnostics)
   int2* lane_best = nullptr;               // local = 1: per-lane (best value, first row)
   int32_t* best_out = nullptr;             // local = 1: the slab's best cell (value, row, col)
   uint32_t epoch = 0;
   cudaEvent_t ev0 = nullptr, ev1 = nullptr;
+  cudaEvent_t ev2 = nullptr;               // after the error-word copy of the last run
   bool ran = false;
   std::string msg;
 };
@@ -157,8 +161,8 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
     case WF_FN_SYNTHETIC:
       if (p->tsize < 0 || p->tsize > 1000000) return fail(c, WF_EINVAL, "tsize=%d out of range 0..1000000", p->tsize);
       if (p->dsize < 0 || p->dsize > 8) return fail(c, WF_EINVAL, "dsize=%d out of range 0..8", p->dsize);
-      if ((long long)rows * cols > 2147483647LL && rows > 46340)
-        return fail(c, WF_EINVAL, "dim too large for the int32 i1 = i*j field");
+      if ((long long)rows * cols > 2147483647LL)   // i1 = i*j of the last cell must fit int32 (R14)
+        return fail(c, WF_EINVAL, "rows*cols=%lld too large for the int32 i1 = i*j field", (long long)rows * cols);
       pl.nf = 2 + p->dsize;
       pl.nbound = p->dsize;
       break;
@@ -336,6 +340,24 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   }
   if (e == cudaSuccess) e = cudaMalloc(&c->err, sizeof(int));
   if (e == cudaSuccess) e = cudaMemset(c->err, 0, sizeof(int));
+  if (e == cudaSuccess) e = cudaMallocHost(&c->err_host, sizeof(int));
+  if (e == cudaSuccess) *c->err_host = 0;
+  // Default watchdog: a dependency wait may legitimately last the pipeline fill up to the last
+  // band -- about nbands x 64 rows of steps, each step costing ~(tsize + 3) x max(dsize, 1) x 8
+  // cycles for the synthetic cell (~100 cycles otherwise) -- so the budget scales with it
+  // (a fixed 2^32 timed out valid large-tsize runs).
+  if (e == cudaSuccess) {
+    if (p->watchdog_cycles) {
+      c->watchdog = p->watchdog_cycles;
+    } else {
+      const double step = p->fn == WF_FN_SYNTHETIC ? 8.0 * (p->tsize + 3) * (p->dsize > 1 ? p->dsize : 1)
+                          : p->fn == WF_FN_NASH  ? 64.0 * p->tsize * p->tsize
+                                                 : 100.0;
+      const double fill = (double)pl.nbands * c->world * 64.0 * step * 4.0;   // x4 margin
+      const double lim = 9.0e18;
+      c->watchdog = (uint64_t)(fill > (double)(1ull << 32) ? (fill < lim ? fill : lim) : (double)(1ull << 32));
+    }
+  }
   if (e == cudaSuccess && L.local) {   // Smith-Waterman best-cell reduction scratch
     e = cudaMalloc(&c->lane_best, (size_t)pl.nbands * pl.warps * 32 * sizeof(int2));
     if (e == cudaSuccess) e = cudaMalloc(&c->best_out, 4 * sizeof(int32_t));
@@ -343,6 +365,7 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   }
   if (e == cudaSuccess) e = cudaEventCreate(&c->ev0);
   if (e == cudaSuccess) e = cudaEventCreate(&c->ev1);
+  if (e == cudaSuccess) e = cudaEventCreateWithFlags(&c->ev2, cudaEventDisableTiming);
   if (e == cudaSuccess) e = cudaDeviceSynchronize();
   if (e != cudaSuccess) {
     st = cuda_fail(nullptr, e, "wf_create scratch");
@@ -358,16 +381,18 @@ wf_status wf_destroy(wf_ctx* c) {
   int prev = -1;
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
-  if (c->ev1) cudaEventSynchronize(c->ev1);
+  if (c->ev2) cudaEventSynchronize(c->ev2);   // the last run and its error-word copy
   if (c->next_ipc_base) cudaIpcCloseMemHandle(c->next_ipc_base);
   if (c->prev_ipc_base) cudaIpcCloseMemHandle(c->prev_ipc_base);
   if (c->base) cudaFree(c->base);
   if (c->err) cudaFree(c->err);
+  if (c->err_host) cudaFreeHost(c->err_host);
   if (c->lane_best) cudaFree(c->lane_best);
   if (c->best_out) cudaFree(c->best_out);
   if (c->trace) cudaFree(c->trace);
   if (c->ev0) cudaEventDestroy(c->ev0);
   if (c->ev1) cudaEventDestroy(c->ev1);
+  if (c->ev2) cudaEventDestroy(c->ev2);
   if (prev >= 0) cudaSetDevice(prev);
   cudaGetLastError();
   delete c;
@@ -378,8 +403,18 @@ wf_status wf_link_local(wf_ctx* prev, wf_ctx* next) {
   if (!prev || !next) return fail(prev, WF_EINVAL, "wf_link_local: NULL context");
   if (next->rank != prev->rank + 1 || next->world != prev->world)
     return fail(prev, WF_EINVAL, "wf_link_local: ranks %d -> %d are not consecutive slabs", prev->rank, next->rank);
-  if (prev->nf != next->nf || prev->p.dim != next->p.dim)
-    return fail(prev, WF_EINVAL, "wf_link_local: contexts describe different problems");
+  if (prev->nf != next->nf || prev->p.dim != next->p.dim || prev->p.fn != next->p.fn ||
+      prev->p.cols != next->p.cols || prev->p.tsize != next->p.tsize || prev->p.dsize != next->p.dsize ||
+      prev->p.local != next->p.local || prev->impl != next->impl || prev->k != next->k ||
+      prev->warps != next->warps || prev->skew != next->skew)
+    return fail(prev, WF_EINVAL, "wf_link_local: contexts describe different problems or tunings");
+  if (prev->c1 != next->c0)
+    return fail(prev, WF_EINVAL, "wf_link_local: slab %d ends at column %d but slab %d starts at %d", prev->rank,
+                prev->c1, next->rank, next->c0);
+  // the slabs' per-run acks and rings are epoch-paired: both must be linked before their first run
+  if (prev->epoch != next->epoch || prev->ran || next->ran)
+    return fail(prev, WF_ESTATE, "wf_link_local: link slabs before their first wf_run (epochs %u / %u)", prev->epoch,
+                next->epoch);
   if (prev->device != next->device) {
     int can = 0;
     cudaDeviceCanAccessPeer(&can, prev->device, next->device);
@@ -440,6 +475,10 @@ static wf_status open_ipc(wf_ctx* c, const void* handle, void** out) {
 
 wf_status wf_connect(wf_ctx* c, const void* prev_handle, const void* next_handle) {
   if (!c) return fail(c, WF_EINVAL, "wf_connect: NULL context");
+  // the slabs' per-run acks and rings are epoch-paired: every rank connects before its first run
+  // (all ranks then issue the same sequence of wf_run calls)
+  if (c->ran || c->epoch != 0)
+    return fail(c, WF_ESTATE, "wf_connect: connect before the first wf_run (this context already ran %u times)", c->epoch);
   if ((c->rank > 0) != (prev_handle != nullptr))
     return fail(c, WF_EINVAL, "wf_connect: rank %d %s a predecessor handle", c->rank, c->rank > 0 ? "needs" : "takes no");
   if ((c->rank < c->world - 1) != (next_handle != nullptr))
@@ -523,6 +562,18 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   L.ack_self = c->ack;
   L.ack_prev = c->ack_prev;
   L.first_slab = c->rank == 0;
+  // a device error of the previous run that has already completed (its error word was copied to
+  // pinned host memory behind it) is reported here, once, without blocking (include/wf.h)
+  if (c->ran && c->reported != c->epoch && cudaEventQuery(c->ev2) == cudaSuccess) {
+    const int w = *reinterpret_cast<volatile int*>(c->err_host);
+    if (((unsigned)w >> 4) == (c->epoch & 0x0FFFFFFFu) && (w & 15) == wfk::DEV_TIMEOUT) {
+      c->reported = c->epoch;
+      return fail(c, WF_ETIMEOUT, "watchdog fired in the previous run (epoch %u; budget %llu cycles per wait)",
+                  c->epoch, (unsigned long long)c->watchdog);
+    }
+  } else {
+    cudaGetLastError();
+  }
   L.epoch = ++c->epoch;
   if ((L.epoch & 0x0FFFFFFFu) == 0) L.epoch = ++c->epoch;   // tag 0 marks "never written"
   L.err = c->err;
@@ -532,7 +583,7 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   }
   if (c->trace) cudaMemsetAsync(c->trace, 0, (size_t)c->nbands * wfk::kTraceSlots * 8, static_cast<cudaStream_t>(cuda_stream));
   L.trace = c->trace;
-  L.watchdog = p.watchdog_cycles ? p.watchdog_cycles : (1ull << 32);
+  L.watchdog = c->watchdog;
 
   int prev = -1;
   cudaGetDevice(&prev);
@@ -542,6 +593,8 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   if (e == cudaSuccess) e = wfk::launch(L, s);
   if (e == cudaSuccess && L.local) e = wfk::launch_sw_best(L, s);   // part of the step: inside the timed events
   if (e == cudaSuccess) e = cudaEventRecord(c->ev1, s);
+  if (e == cudaSuccess) e = cudaMemcpyAsync(c->err_host, c->err, sizeof(int), cudaMemcpyDeviceToHost, s);
+  if (e == cudaSuccess) e = cudaEventRecord(c->ev2, s);
   if (prev >= 0 && prev != c->device) cudaSetDevice(prev);
   if (e != cudaSuccess) return cuda_fail(c, e, "wf_run launch");
   c->ran = true;
@@ -556,9 +609,13 @@ wf_status wf_sync(wf_ctx* c) {
   int w = 0;
   e = cudaMemcpy(&w, c->err, sizeof w, cudaMemcpyDeviceToHost);
   if (e != cudaSuccess) return cuda_fail(c, e, "wf_sync error word");
-  if (((unsigned)w >> 4) == (c->epoch & 0x0FFFFFFFu) && (w & 15) == wfk::DEV_TIMEOUT)
-    return fail(c, WF_ETIMEOUT, "watchdog: a dependency wait exceeded %llu cycles (run epoch %u)",
-                (unsigned long long)(c->p.watchdog_cycles ? c->p.watchdog_cycles : (1ull << 32)), c->epoch);
+  if (((unsigned)w >> 4) == (c->epoch & 0x0FFFFFFFu) && (w & 15) == wfk::DEV_TIMEOUT) {
+    c->reported = c->epoch;
+    return fail(c, WF_ETIMEOUT,
+                "watchdog: a dependency wait exceeded %llu cycles (run epoch %u; linked slabs must issue the same "
+                "sequence of wf_run calls)",
+                (unsigned long long)c->watchdog, c->epoch);
+  }
   return WF_OK;
 }
 

@@ -614,7 +614,7 @@ cudaError_t launch(const SweepLaunch& L, cudaStream_t s, size_t smem) {
 template <int K, int WARPS, bool LOCAL>
 Variant make() {
   return Variant{WF_FN_SEQCMP, LOCAL ? 1 : 0, K, WARPS, 1, (WARPS + 1) * 32, Smem<K, WARPS>::bytes,
-                 reinterpret_cast<const void*>(nw8_kernel<K, WARPS, LOCAL, kU>), &launch<K, WARPS>, 8};
+                 reinterpret_cast<const void*>(nw8_kernel<K, WARPS, LOCAL, kU>), &launch<K, WARPS>, 8, {}};
 }
 
 }  // namespace nw8

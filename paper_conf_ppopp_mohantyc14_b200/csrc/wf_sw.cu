@@ -92,7 +92,8 @@ Variant make_sw() {
   using S = NwSmem<K, W, D, U>;
   // dsize = 1 marks the local (Smith-Waterman) variant of SEQCMP in the variant table
   return Variant{WF_FN_SEQCMP, 1, K, W, D, (W + 2) * 32, S::bytes,
-                 reinterpret_cast<const void*>(nw_kernel<K, W, D, U, true, true>), &launch_sw<K, W, D, U>, 4};
+                 reinterpret_cast<const void*>(nw_kernel<K, W, D, U, true, true>), &launch_sw<K, W, D, U>, 4,
+                 {reinterpret_cast<const void*>(nw_kernel<K, W, D, U, false, true>)}};
 }
 
 }  // namespace

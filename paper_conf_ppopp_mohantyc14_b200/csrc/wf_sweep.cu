@@ -127,7 +127,7 @@ Variant make_nw_variant() {
   using S = NwSmem<K, W, D, U>;
   return Variant{WF_FN_SEQCMP, 0, K, W, D, (W + 2) * 32, S::bytes,
                  reinterpret_cast<const void*>(nw_kernel<K, W, D, U, true>),
-                 &launch_nw<K, W, D, U>, 4};
+                 &launch_nw<K, W, D, U>, 4, {reinterpret_cast<const void*>(nw_kernel<K, W, D, U, false>)}};
 }
 
 template <int W>
@@ -151,7 +151,8 @@ cudaError_t launch_nash(const SweepLaunch& L, cudaStream_t s, size_t smem) {
 template <int W>
 Variant make_nash_variant() {
   return Variant{WF_FN_NASH, 0, 1, W, 1, (W + 1) * 32, NashSmem<W>::fixed_bytes,
-                 reinterpret_cast<const void*>(nash_kernel<W, 16>), &launch_nash<W>, 4};
+                 reinterpret_cast<const void*>(nash_kernel<W, 16>), &launch_nash<W>, 4,
+                 {reinterpret_cast<const void*>(nash_kernel<W, 0>)}};
 }
 
 // --- the compiled variant set -------------------------------------------------------
@@ -239,12 +240,24 @@ int occupancy(const SweepLaunch& L, int smem) {
     cudaGetLastError();
     return 0;
   }
-  int blocks = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, v->kernel, v->threads, smem) != cudaSuccess) {
-    cudaGetLastError();
-    return 0;
+  // every instantiation launch() may pick must be co-resident at the grid size (all CTAs spin
+  // on each other): the minimum over the variant's kernel and its alternatives
+  int best = -1;
+  for (int i = -1; i < 4; ++i) {
+    const void* k = i < 0 ? v->kernel : v->alt[i];
+    if (!k) continue;
+    if (cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem) != cudaSuccess) {
+      cudaGetLastError();
+      return 0;
+    }
+    int blocks = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, k, v->threads, smem) != cudaSuccess) {
+      cudaGetLastError();
+      return 0;
+    }
+    best = best < 0 ? blocks : (blocks < best ? blocks : best);
   }
-  return blocks;
+  return best < 0 ? 0 : best;
 }
 
 cudaError_t launch(const SweepLaunch& L, cudaStream_t s) {

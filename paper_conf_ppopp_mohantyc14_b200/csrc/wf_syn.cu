@@ -593,15 +593,26 @@ cudaError_t launch_syn_ps(const SweepLaunch& L, cudaStream_t s, size_t smem) {
 template <int DS>
 Variant make_syn_ps() {
   using S = SynSmem<DS, 1, 1>;
-  return Variant{WF_FN_SYNTHETIC, DS, 1, 1, 1, (DS + 1) * 32, S::bytes,
-                 reinterpret_cast<const void*>(syn_ps_kernel<DS, 0>), &launch_syn_ps<DS>, 8};
+  Variant v{WF_FN_SYNTHETIC, DS, 1, 1, 1, (DS + 1) * 32, S::bytes,
+            reinterpret_cast<const void*>(syn_ps_kernel<DS, 0>), &launch_syn_ps<DS>, 8, {}};
+  if constexpr (DS == 5) {
+    v.alt[0] = reinterpret_cast<const void*>(syn_ps_kernel<DS, 100>);
+    v.alt[1] = reinterpret_cast<const void*>(syn_ps_kernel<DS, 1000>);
+  }
+  return v;
 }
 
 template <int DS, int K, int W>
 Variant make_syn() {
   using S = SynSmem<DS, K, W>;
-  return Variant{WF_FN_SYNTHETIC, DS, K, W, 1, (W + 1 + syn_pad(DS)) * 32, S::bytes,
-                 reinterpret_cast<const void*>(syn_kernel<DS, K, W, 0>), &launch_syn<DS, K, W>, 7};
+  Variant v{WF_FN_SYNTHETIC, DS, K, W, 1, (W + 1 + syn_pad(DS)) * 32, S::bytes,
+            reinterpret_cast<const void*>(syn_kernel<DS, K, W, 0>), &launch_syn<DS, K, W>, 7, {}};
+  if constexpr (K == 1 && (DS == 1 || DS == 5)) {   // the compile-time tsize kernels launch_syn picks
+    v.alt[0] = reinterpret_cast<const void*>(syn_kernel<DS, K, W, 10>);
+    v.alt[1] = reinterpret_cast<const void*>(syn_kernel<DS, K, W, 100>);
+    v.alt[2] = reinterpret_cast<const void*>(syn_kernel<DS, K, W, 1000>);
+  }
+  return v;
 }
 
 #define WF_SYN7(DS) make_syn<DS, 1, 1>(), make_syn<DS, 1, 2>(), make_syn<DS, 1, 4>(), make_syn<DS, 2, 2>()

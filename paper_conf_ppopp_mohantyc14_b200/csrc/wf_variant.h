@@ -13,7 +13,9 @@ struct Variant {
   size_t smem;
   const void* kernel;  // __global__ function pointer (for occupancy queries)
   cudaError_t (*launch)(const SweepLaunch&, cudaStream_t, size_t);
-  int impl;            // kernel generation (SEQCMP: 4 = block hand-offs, 7 = per-row hand-offs)
+  int impl;            // kernel generation (SEQCMP: 4 = block hand-offs, 8 = lane pipeline)
+  const void* alt[4];  // other instantiations launch() may pick for this variant (e.g. compile-time
+                       // tsize); occupancy() takes the minimum over kernel and alt[]
 };
 
 // SEQCMP v8 variants (wf_nw8.cu): global (dsize 0) and local / Smith-Waterman (dsize 1)

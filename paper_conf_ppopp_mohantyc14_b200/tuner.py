@@ -41,12 +41,19 @@ def predict_log_ms(x, tree=None) -> float:
 
 def suggest(fn: str, dim: int, tsize: int = 0, dsize: int = 0) -> dict:
     """Wavefront keyword arguments (lane_cols, warps, skew, kernel) of the predicted-fastest
-    variant among those the model was trained on for this function."""
+    variant among those the model was trained on for this function that the library accepts
+    for this instance (wf_query: compiled, fits shared memory -- e.g. a wide synthetic variant
+    with many float items does not).  Falls back to the library defaults (all zero)."""
+    from .wf import query   # host-side wf_query only
     m = _model()
-    best = None
-    for k, w, d, impl in m["candidates"][fn]:
-        p = predict_log_ms(features(fn, dim, tsize, dsize, k, w, d, impl), m["tree"])
-        if best is None or p < best[0]:
-            best = (p, k, w, d, impl)
-    _, k, w, d, impl = best
-    return {"lane_cols": k, "warps": w, "skew": d, "kernel": impl}
+    ranked = sorted((predict_log_ms(features(fn, dim, tsize, dsize, k, w, d, impl), m["tree"]), k, w, d, impl)
+                    for k, w, d, impl in m["candidates"][fn])
+    extra = {"tsize": tsize, "dsize": dsize} if fn != "seqcmp" else {}
+    for _, k, w, d, impl in ranked:
+        try:
+            lay = query(fn, dim, lane_cols=k, warps=w, skew=d, kernel=impl, **extra)
+        except Exception:   # noqa: BLE001 -- WF_EUNSUPPORTED / WF_EINVAL: not buildable here
+            continue
+        if (lay.lane_cols, lay.warps, lay.skew) == (k, w, d):
+            return {"lane_cols": k, "warps": w, "skew": d, "kernel": impl}
+    return {"lane_cols": 0, "warps": 0, "skew": 0, "kernel": 0}

@@ -30,7 +30,9 @@ def test_tree_evaluator_matches_sklearn_fit_on_the_sweep():
 
 @pytest.mark.parametrize("fn,dim,tsize,dsize", [("seqcmp", 32768, 0, 0), ("seqcmp", 3000, 0, 0),
                                                 ("synthetic", 16384, 10, 1), ("synthetic", 2048, 100, 1),
-                                                ("synthetic", 8000, 500, 4), ("nash", 4096, 16, 4)])
+                                                ("synthetic", 8000, 500, 4), ("nash", 4096, 16, 4),
+                                                ("synthetic", 16384, 100, 8), ("synthetic", 16384, 1000, 8),
+                                                ("synthetic", 4096, 1000, 6), ("synthetic", 4096, 1000, 7)])
 def test_suggestions_are_compiled_variants(fn, dim, tsize, dsize):
     kw = tuner.suggest(fn, dim, tsize, dsize)
     assert set(kw) == {"lane_cols", "warps", "skew", "kernel"}

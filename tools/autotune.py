@@ -9,10 +9,12 @@ The paper's tunables (cpu-tile, band, gpu-count, gpu-tile, halo) map onto this b
 (DESIGN.md §6-7):
   * tile      -> lane_cols K (columns per lane) x warps W (the CTA band is 32*K*W columns),
   * strip     -> lane skew D (rows between neighbouring lanes) and, for sequence comparison,
-                 the hand-off kernel (WF_NW_IMPL 4 = U-row blocks, 7 = per-row LL words),
-  * gpu-count -> column slabs; on one physical GPU the slab chain is exercised with
-                 device_share (virtual slabs) -- correct but not a speed-up, so the harness
-                 records it as a scaling point only when more than one GPU is visible.
+                 the kernel generation (wf_params.kernel 8 = lockstep lane pipeline, 4 = U-row
+                 block hand-offs),
+  * gpu-count -> column slabs (--slabs G...): G slabs linked by the per-row P2P hand-off.  On one
+                 physical GPU they are virtual slabs sharing its SMs (device_share) -- a
+                 correctness and hand-off-cost point, not a speed-up; with G visible GPUs each slab
+                 gets its own device.
 Every point is first checked against the CPU oracle on a small instance of the same
 function (parity gate: a point that is wrong is discarded, never timed), then timed on the
 config's full size with CUDA events (median of --reps runs after 3 warm-ups).  The winner
@@ -36,13 +38,13 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
 import oracle  # noqa: E402  (parity gate only; the timed path never touches it)
 import workloads  # noqa: E402
-from paper_conf_ppopp_mohantyc14_b200.wf import Wavefront  # noqa: E402
+from paper_conf_ppopp_mohantyc14_b200.wf import LocalSlabs, Wavefront, query  # noqa: E402
 
-# impl = wf_params.kernel: 4 = first generation (NW v4 / generic synthetic sweep),
-# 7 = second generation (NW v7 / wf_syn), 8 = plane-split wf_syn (synthetic, dsize >= 2, k = w = d = 1);
-# Nash has one kernel (0)
+# impl = wf_params.kernel: SEQCMP 8 = lockstep lane pipeline (wf_nw8.cu), 4 = block hand-offs (v4);
+# SYNTHETIC 7 = wf_syn, 4 = generic sweep, 8 = plane-split wf_syn (dsize >= 2, k = w = d = 1);
+# Nash has one kernel (0).  Combinations a generation does not compile are skipped (wf_query).
 SEARCH = {
-    "seqcmp": {"k": [2, 4, 8], "w": [1, 2, 4], "d": [1, 2], "impl": [4, 7]},
+    "seqcmp": {"k": [1, 2, 4, 8], "w": [1, 2, 4, 8], "d": [1, 2], "impl": [8, 4]},
     "synthetic": {"k": [1, 2], "w": [1, 2, 4], "d": [1, 2], "impl": [7, 4, 8]},
     "nash": {"k": [1], "w": [1, 2, 4, 8], "d": [1], "impl": [0]},
 }
@@ -124,6 +126,56 @@ def time_point(cfg, k, w, d, impl, devin, reps):
         return statistics.median(ms), wf.layout.nbands
 
 
+def compiled(cfg, k, w, d, impl):
+    """Does the library build this (fn, tuning, generation)?  (host-side wf_query; no GPU work)"""
+    try:
+        lay = query(cfg.fn, cfg.dim, lane_cols=k, warps=w, skew=d, kernel=impl, **fn_kw(cfg))
+    except Exception:  # noqa: BLE001 -- WF_EUNSUPPORTED / WF_EINVAL
+        return False
+    return (lay.lane_cols, lay.warps, lay.skew) == (k, w, d)
+
+
+def time_slabs(cfg, k, w, d, impl, host, G, reps):
+    """G column slabs of the same grid linked by the per-row P2P hand-off (virtual slabs on one GPU)."""
+    ngpu = torch.cuda.device_count()
+    devices = [g % ngpu for g in range(G)]
+    ls = LocalSlabs(cfg.fn, cfg.dim, G, devices=devices, lane_cols=k, warps=w, skew=d, kernel=impl, **fn_kw(cfg))
+    try:
+        per = [inputs_for(cfg.fn, cfg.dim, cfg.dsize, torch.device("cuda", s.device))[1] for s in ls.slabs]
+        outs = None
+        for _ in range(3):
+            outs = ls.run(per, outs)
+        ls.sync()
+        ms = []
+        for _ in range(reps):
+            for dv in set(devices):
+                torch.cuda.synchronize(dv)
+            t0 = time.perf_counter()
+            outs = ls.run(per, outs)
+            ls.sync()
+            ms.append((time.perf_counter() - t0) * 1e3)
+        return statistics.median(ms)
+    finally:
+        ls.close()
+
+
+def sweep_slabs(cfg, reps, slabs):
+    """The gpu-count axis: the config's default tuning on G slabs (wall clock around the linked runs)."""
+    host, _ = inputs_for(cfg.fn, 16, cfg.dsize, torch.device("cuda", 0))
+    recs = []
+    for G in slabs:
+        rec = {"slabs": G, "visible_gpus": torch.cuda.device_count(),
+               "placement": "virtual (one GPU)" if torch.cuda.device_count() < G else "one GPU per slab"}
+        try:
+            ms = time_slabs(cfg, 0, 0, 0, 0, host, G, reps)
+            rec.update(ms=round(ms, 4), gcups=round(cfg.dim * cfg.dim / ms / 1e6, 3))
+        except Exception as e:  # noqa: BLE001
+            rec["error"] = str(e)[:160]
+        recs.append(rec)
+        print(json.dumps(rec), flush=True)
+    return recs
+
+
 def tune(cfg, reps, small, budget_s):
     dev = torch.device("cuda", 0)
     _, devin = inputs_for(cfg.fn, cfg.dim, cfg.dsize, dev)
@@ -131,7 +183,7 @@ def tune(cfg, reps, small, budget_s):
     points = []
     t_start = time.time()
     for impl, k, w, d in itertools.product(sp["impl"], sp["k"], sp["w"], sp["d"]):
-        if cfg.fn == "seqcmp" and impl == 7 and d != 1:
+        if not compiled(cfg, k, w, d, impl):
             continue
         if time.time() - t_start > budget_s:
             points.append({"impl": impl, "k": k, "w": w, "d": d, "skipped": "time budget"})
@@ -162,15 +214,21 @@ GRID = ([("seqcmp", d, 0, 0) for d in (1024, 2048, 4096, 8192, 16384, 32768)]
         + [("nash", d, 16, 4) for d in (1024, 2048, 4096)])
 
 
-def sweep_grid(reps, out):
+def sweep_grid(reps, out, only_fn=None):
+    """Time every compiled variant on every GRID instance; with only_fn, re-sweep that function and
+    keep the other functions' points of the existing file."""
     dev = torch.device("cuda", 0)
     recs = []
+    if only_fn and os.path.exists(out):
+        recs = [p for p in json.load(open(out))["points"] if p["fn"] != only_fn]
     for fn, dim, tsize, dsize in GRID:
+        if only_fn and fn != only_fn:
+            continue
         cfg = workloads.Config(f"{fn}-{dim}-{tsize}-{dsize}", fn, dim, tsize=tsize, dsize=dsize)
         _, devin = inputs_for(fn, dim, dsize, dev)
         sp = SEARCH[fn]
         for impl, k, w, d in itertools.product(sp["impl"], sp["k"], sp["w"], sp["d"]):
-            if fn == "seqcmp" and impl == 7 and d != 1:
+            if not compiled(cfg, k, w, d, impl):
                 continue
             rec = {"fn": fn, "dim": dim, "tsize": tsize, "dsize": dsize, "impl": impl, "k": k, "w": w, "d": d}
             try:
@@ -194,9 +252,20 @@ def main():
     ap.add_argument("--small", type=int, default=300, help="parity-gate instance size")
     ap.add_argument("--budget-s", type=float, default=240.0, help="per-config time budget")
     ap.add_argument("--out", default="")
+    ap.add_argument("--grid-fn", default=None, choices=[None, "seqcmp", "synthetic", "nash"],
+                    help="with --grid: re-sweep one function, keep the others' points")
+    ap.add_argument("--slabs", default="", help="gpu-count axis, e.g. 1,2,4,8 (column slabs of --config)")
     a = ap.parse_args()
     if a.grid:
-        sweep_grid(a.reps, a.out or os.path.join(ROOT, "profiles", "tuner_sweep.json"))
+        sweep_grid(a.reps, a.out or os.path.join(ROOT, "profiles", "tuner_sweep.json"), a.grid_fn)
+        return
+    if a.slabs:
+        cfg = workloads.CONFIGS[a.config]
+        res = {"config": cfg.name, "fn": cfg.fn, "dim": cfg.dim, "reps": a.reps,
+               "device": torch.cuda.get_device_name(0), "points": sweep_slabs(cfg, a.reps, [int(g) for g in a.slabs.split(",")])}
+        out = a.out or os.path.join(ROOT, "profiles", f"autotune_slabs_{cfg.name}.json")
+        with open(out, "w") as f:
+            json.dump(res, f, indent=1)
         return
     names = sorted(workloads.CONFIGS) if a.all else [a.config]
     for n in names:
