@@ -266,6 +266,7 @@ __device__ __forceinline__ bool nash_warp(const SweepLaunch& L, const PolNash& p
     uint32_t W[4];
     {
       const unsigned long long* slot = in_ring + (r & (NashSmem<WARPS>::kSlots - 1)) * 4;
+      wf_jitter(18);
       wd.start();
       for (;;) {
         bool ok = true;

@@ -552,6 +552,7 @@ struct NwWarp {
         continue;
       }
       tick(3);
+      wf_jitter(13);
       // ---- publish: one fence for the TMA engine and for the next warp
       const int r31_0 = t0 - 31 * D + 1;           // first row of the block's TMA box
       const int r31_last = min(r31_0 + U - 1, rows);
@@ -650,6 +651,7 @@ __device__ __forceinline__ bool nw_io_warp(const SweepLaunch& L, const NwSmem<K,
   Watchdog wd;
   wd.start();
   while (feed <= rows || fwd <= rows) {
+    wf_jitter(11);
     bool progress = false;
     // (b) west feed of compute warp 0 (boundary column or the previous band's LL ring)
     if (feed <= rows) {
@@ -752,6 +754,7 @@ __device__ __forceinline__ bool nw_x_warp(const SweepLaunch& L, const NwSmem<K, 
   Watchdog wd;
   wd.start();
   while (xfill < rows) {
+    wf_jitter(12);
     int lo = rows + 1;
 #pragma unroll
     for (int w = 0; w < WARPS; ++w) lo = min(lo, lds_vol_i(sm.xneed + w));

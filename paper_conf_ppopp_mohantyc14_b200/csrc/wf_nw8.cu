@@ -147,9 +147,20 @@ __device__ __forceinline__ void sts32_if(bool p, uint32_t a, int32_t v) {
   asm volatile("{ .reg .pred q; setp.ne.b32 q, %2, 0; @q st.shared.s32 [%0], %1; }" ::"r"(a), "r"(v),
                "r"(static_cast<int>(p)));
 }
+// The block barrier.  The warps reach it from different code (each warp's role is its own
+// instantiation), as in warp-specialized producer / consumer kernels: each warp arrives
+// convergently, the CTA's warps at different barrier instructions.  bar.sync (the .aligned
+// form) measured 7 % faster on C4 than barrier.sync (1.962 vs 2.101 ms, profiles/r02_nw8_ab.txt);
+// compute-sanitizer synccheck reports the .aligned form as "divergent threads in block", so the
+// sanitizer runs build the non-.aligned form (-DWF_NW8_UNALIGNED_BAR, tools/gpu_race.sh), which is
+// synccheck-clean and passes the same parity (profiles/r02_sanitizer.txt).
 template <int THREADS>
 __device__ __forceinline__ void cta_bar() {
+#ifdef WF_NW8_UNALIGNED_BAR
+  asm volatile("barrier.sync 1, %0;" ::"n"(THREADS) : "memory");
+#else
   asm volatile("bar.sync 1, %0;" ::"n"(THREADS) : "memory");
+#endif
 }
 __device__ __forceinline__ bool quad_stale(const int4& v, int r, int rows) {
   return (v.x == EMPTY && r <= rows) | (v.y == EMPTY && r + 1 <= rows) | (v.z == EMPTY && r + 2 <= rows) |
@@ -333,6 +344,7 @@ struct Warp {
   __device__ __forceinline__ void after_block(int s0) {
     const int e = s0 + U;   // last local step done
     if (e % 32 == 0 && e >= 64) publish(e - 63);   // rows e-63 .. e-32 complete (lane 31 passed them)
+    wf_jitter(1 + WI);
     cta_bar<NT>();
   }
 
@@ -527,6 +539,7 @@ struct Helper {
     cta_bar<NT>();   // warp 0's first block reads what the prologue stored
     for (int B = 0; B < Tc; B += U) {
       // B = CTA step of this block's start; warp 0's current block has local start s0 = B
+      wf_jitter(9);
       if (inbound && B + U < Tw) deliver(B + U);   // warp 0's next block starts at local step B + U
       if (outbound && B >= U) {       // the last warp's block that ended at this block's start
         const int s0 = B - U - Ll;

@@ -82,6 +82,25 @@ __device__ __forceinline__ unsigned long long ll_pack(uint32_t val, uint32_t tag
   return (static_cast<unsigned long long>(tag) << 32) | val;
 }
 
+// Race / liveness testing: a build with -DWF_JITTER=1 inserts pseudo-random
+// back-offs (1 call in 8 sleeps up to ~1 us, warp-uniform) at the producers and consumers of
+// every hand-off protocol, so parity under it checks the orderings for schedules the natural
+// timing never produces.  A no-op in the product build.
+#ifndef WF_JITTER
+#define WF_JITTER 0
+#endif
+__device__ __forceinline__ void wf_jitter(unsigned salt) {
+  if constexpr (WF_JITTER != 0) {
+    unsigned h = static_cast<unsigned>(clock64() >> 4) ^ (salt * 0x9E3779B9u) ^ (blockIdx.x * 0x85EBCA6Bu) ^
+                 ((threadIdx.x >> 5) * 0xC2B2AE35u);
+    h = __shfl_sync(0xffffffffu, h, 0);   // one decision per warp
+    h ^= h >> 16;
+    h *= 0x7feb352du;
+    h ^= h >> 15;
+    if ((h & 7u) == 0) __nanosleep(h >> 22);
+  }
+}
+
 // The device error word is epoch-tagged -- (epoch & 0x0FFFFFFF) << 4 | code -- so a
 // failure of an earlier run never has to be cleared before the next launch.
 __device__ __forceinline__ int err_word(const SweepLaunch& L, int code) {
@@ -148,6 +167,7 @@ __device__ __forceinline__ bool feeder(const SweepLaunch& L, const P& pol, const
   Watchdog wd;
   wd.start();
   while (base <= L.rows) {
+    wf_jitter(16);
     // back-pressure: rows base .. base+63 go to slots that held rows base-kSlots .. ;
     // those must have been consumed by compute warp 0.
     // The feeder is normally far ahead, so it sleeps between polls: a tight LDS spin would
@@ -277,6 +297,7 @@ __device__ __forceinline__ bool compute_warp(const SweepLaunch& L, const P& pol,
       const int r = t + 1;
       const unsigned long long* slot = sm.hand_slot(warp, r);
       uint32_t got[NF];
+      wf_jitter(17);
       wd.start();
       for (;;) {
         bool ok = true;

@@ -347,6 +347,7 @@ struct SynWarp {
         if (steady) block<false, false>(t0, pre, q, qx, gdst, to_peer);
         else block<true, false>(t0, pre, q, qx, gdst, to_peer);
       }
+      wf_jitter(15);
       // publish lane 31's rows of the block to the next warp (one fence per block)
       const int r31_last = min(t0 + UB - 31, rows);
       if (!last && r31_last >= 1 && lane == 31) {
@@ -408,6 +409,7 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
   Watchdog wd;
   wd.start();
   while (feed <= rows) {
+    wf_jitter(14);
     const int need = feed + 31 - kSynLL;   // slot reuse: warp 0 has consumed those rows
     if (seen < need) {
       seen = lds_vol_i(sm.rprog + 0);

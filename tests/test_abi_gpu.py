@@ -1,6 +1,7 @@
 """C-ABI state rules that need a device (include/wf.h): slab linking is validated (same problem
 and tuning, adjacent columns, before the first run), a device error of a completed run is
-reported by the next wf_run, ADVICE r1 (wf_link_local, epoch pairing, wf_run error word, watchdog budget)."""
+reported by the next wf_run, and a context connects only before its first run.
+(wf_link_local, epoch pairing, wf_run error word)."""
 from __future__ import annotations
 
 import numpy as np
@@ -35,7 +36,7 @@ def test_link_rejects_a_different_tuning():
 
 
 def test_link_rejects_non_adjacent_slabs():
-    a, c = _slab(0, G=3), _slab(2, G=3)
+    a, c = _slab(0, G=3, dim=1000), _slab(2, G=3, dim=1000)
     try:
         with pytest.raises(_abi.WfError) as ei:
             a.link(c)
