@@ -51,15 +51,26 @@ SMS = 148
 FP32_LANES_PER_SM = 128      # B200_PROFILING.md unit counts: 4 SMSPs x 32 FP32 lanes
 CELL_CHAIN_CYC = 4.12        # dependent FADD/FMUL/FFMA latency, profiles/r01_microbench.txt (lat_ffma_cyc)
 NASH_INT_OPS_PER_CELL = 5120  # n=16: 2 n^2 payoff hashes x ~8 int ops + n^2 best-response tests x ~4
+NW_OPS_PER_CELL = 3          # s(x_i, y_j) lookup, NW + s, 3-way max with N - g / W - g (one DPX VIADDMNMX)
+DPX_LANES_PER_SM = 64        # DPX issues at half rate (profiles/r01_microbench.txt mb10)
+DPX_CHAIN_CYC = 4.12         # dependent VIADDMNMX latency (lat_viaddmax_cyc)
+LANE_HOP_CYC = 29.76         # SHFL + dependent DPX, one lane-to-lane hand-off (lat_shfl_plus_viaddmax_cyc)
+NASH_CELL_CHAIN_CYC = 1558.1 # measured serial cost of one Nash cell on a 1-column grid (profiles/r02_chain.txt)
 
 
-def roofline_model(cfg, slab_cells, avg_launch_ms, world):
-    """The dominant kernel's roof for this config.
+def roofline_model(cfg, slab_cells, avg_launch_ms, world, lane_cols=1):
+    """The dominant kernel's roofs for this config (DESIGN.md §5.5 / §11).
 
-    seqcmp and low-tsize synthetic: HBM, algorithmic bytes = cells x B/cell (each output cell
-    written once).  High-tsize synthetic and Nash: plain FP32 / INT32 ALU issue, algorithmic
-    ops = cells x ops/cell.  The bound is the slower roof; both are reported, plus the
-    dependency-chain (latency) roof of the 2*dim-1 anti-diagonals as a diagnostic."""
+    Three roofs, each in GCUPS per GPU:
+      hbm      -- algorithmic bytes = cells x B/cell (every output cell written once);
+      alu      -- algorithmic ops = cells x ops/cell at the issue rate of the unit that runs them;
+      latency  -- the dependency chain: the 2*dim-1 anti-diagonals each need one full cell after
+                  their predecessor (cell chain cycles at sm_max_mhz); no schedule can beat it.
+    `binding` names the lowest of the three.  `bound`/`frac` stay the HBM-or-ALU roof of the
+    metric (BASELINE.json: "% of HBM roofline"), so rounds stay comparable.  For seqcmp the
+    lane-pipeline schedule we ship adds a fourth, schedule-specific figure (`pipeline_roof`):
+    a K-column lane needs >= one SHFL + DPX hand-off per row step, so
+    T >= (rows + cols/K - 1) x 29.76 cycles."""
     hbm_peak, hbm_src = load_peaks()
     try:
         with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
@@ -71,36 +82,48 @@ def roofline_model(cfg, slab_cells, avg_launch_ms, world):
     bpc = cfg.bytes_per_cell()
     hbm = {"achieved": slab_cells * bpc / secs / 1e9, "peak": hbm_peak, "unit": "GB/s",
            "roof_gcups": hbm_peak / bpc, "algorithmic_bytes_per_launch": slab_cells * bpc, "peak_source": hbm_src}
+    src_units = f"{SMS} SMs x {{}} lanes x {mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)"
     if cfg.fn == "seqcmp":
-        alu = None
+        ops, kind, lanes = NW_OPS_PER_CELL, "INT32/DPX", DPX_LANES_PER_SM
+        chain = DPX_CHAIN_CYC
+    elif cfg.fn == "synthetic":
+        ops = 2 + cfg.dsize * (cfg.tsize + 3)   # c = (u*v)*2^-12; per item 2 FADD + FMUL + tsize FFMA
+        chain = CELL_CHAIN_CYC * (cfg.tsize + 3) if cfg.dsize else CELL_CHAIN_CYC
+        kind, lanes = "FP32", FP32_LANES_PER_SM
     else:
-        if cfg.fn == "synthetic":
-            ops = 2 + cfg.dsize * (cfg.tsize + 3)   # c = (u*v)*2^-12; per item 2 FADD + FMUL + tsize FFMA
-            chain = CELL_CHAIN_CYC * (cfg.tsize + 3) if cfg.dsize else CELL_CHAIN_CYC
-            kind = "FP32"
-        else:
-            ops = NASH_INT_OPS_PER_CELL
-            chain = None
-            kind = "INT32"
-        peak_ops = SMS * FP32_LANES_PER_SM * ghz   # G lane-ops/s
-        alu = {"achieved": slab_cells * ops / secs / 1e9, "peak": peak_ops, "unit": f"G{kind} op/s",
-               "ops_per_cell": ops, "roof_gcups": peak_ops / ops,
-               "peak_source": f"{SMS} SMs x {FP32_LANES_PER_SM} lanes x {mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)"}
-    if alu is not None and alu["roof_gcups"] < hbm["roof_gcups"]:
+        ops, kind, lanes = NASH_INT_OPS_PER_CELL, "INT32", FP32_LANES_PER_SM
+        chain = NASH_CELL_CHAIN_CYC
+    peak_ops = SMS * lanes * ghz   # G lane-ops/s
+    alu = {"achieved": slab_cells * ops / secs / 1e9, "peak": peak_ops, "unit": f"G{kind} op/s",
+           "ops_per_cell": ops, "roof_gcups": peak_ops / ops, "peak_source": src_units.format(lanes)}
+    if alu["roof_gcups"] < hbm["roof_gcups"]:
         dom, bound = alu, "alu"
     else:
         dom, bound = hbm, "hbm"
     out = {"bound": bound, "achieved": dom["achieved"], "peak": dom["peak"], "unit": dom["unit"],
            "frac": dom["achieved"] / dom["peak"], "peak_source": dom["peak_source"], "avg_launch_ms": avg_launch_ms,
-           "roof_gcups_per_gpu": dom["roof_gcups"], "hbm": hbm}
-    if alu is not None:
-        out["alu"] = alu
-    if cfg.fn == "synthetic" and cfg.dsize:
+           "roof_gcups_per_gpu": dom["roof_gcups"], "hbm": hbm, "alu": alu}
+    achieved_gcups = slab_cells / secs / 1e9
+    roofs = {"hbm": hbm["roof_gcups"], "alu": alu["roof_gcups"]}
+    if chain is not None:
         diag = 2 * cfg.dim - 1
         lat_gcups = cfg.dim * cfg.dim / (diag * chain / (ghz * 1e9)) / 1e9
+        roofs["latency"] = lat_gcups
         out["latency_roof"] = {"gcups": lat_gcups, "cycles_per_cell_on_chain": chain, "anti_diagonals": diag,
-                               "note": "dependency chain: every anti-diagonal needs one full cell (tsize-deep "
-                                       "FMA chain) after its predecessor; no schedule can beat it"}
+                               "frac": cfg.dim * cfg.dim / secs / 1e9 / lat_gcups if world == 1 else None,
+                               "note": "dependency chain: every anti-diagonal needs one full cell after its "
+                                       "predecessor; no schedule can beat it"}
+    if cfg.fn == "seqcmp":
+        steps = cfg.dim + -(-cfg.dim // max(1, lane_cols)) - 1
+        pipe_s = steps * LANE_HOP_CYC / (ghz * 1e9)
+        pipe_gcups = cfg.dim * cfg.dim / pipe_s / 1e9
+        out["pipeline_roof"] = {"gcups": pipe_gcups, "row_steps": steps, "cycles_per_step": LANE_HOP_CYC,
+                                "lane_cols": lane_cols,
+                                "frac": cfg.dim * cfg.dim / secs / 1e9 / pipe_gcups if world == 1 else None,
+                                "note": "the shipped lane-pipeline schedule: rows + cols/K - 1 row steps, each "
+                                        ">= one SHFL + dependent DPX hand-off (profiles/r01_microbench.txt)"}
+    out["binding"] = min(roofs, key=roofs.get)
+    out["binding_frac"] = achieved_gcups / roofs[out["binding"]] if world == 1 else None
     if bound == "hbm":
         out["algorithmic_bytes_per_launch"] = hbm["algorithmic_bytes_per_launch"]
     return out
@@ -382,13 +405,15 @@ def run_ours(args, cfg):
         torch.cuda.synchronize()
         gms = g0.elapsed_time(g1) / reps
         grid_e2e = {"value": total_cells / (gms * 1e-3) / 1e9, "unit": UNIT, "ms_per_step": gms,
-                    "d2h_bytes_per_step": int(footprint), "h2d_bytes_per_step": h2d}
+                    "d2h_bytes_per_step": int(footprint), "h2d_bytes_per_step": h2d,
+                    "note": "the paper's timing (whole program incl. copying the full score grid back): "
+                            "bound by the PCIe D2H of the grid, not by the sweep"}
         del host_grid
 
-    roof = roofline_model(cfg, slab_cells, avg_launch_ms, world)
+    roof = roofline_model(cfg, slab_cells, avg_launch_ms, world, lay.lane_cols)
     key = f"{cfg.name}_k{lay.lane_cols}w{lay.warps}d{lay.skew}"
     roof["traffic"] = load_traffic(key)
-    roof["kernel"] = {"seqcmp": "wfk::nw_kernel", "synthetic": "wfk::syn_kernel", "nash": "wfk::nash_kernel"}[cfg.fn]
+    roof["kernel"] = {"seqcmp": ("wfk::nw8::nw8_kernel" if w.params.kernel in (0, 8) and lay.skew == 1 else "wfk::nw_kernel"), "synthetic": "wfk::syn_kernel", "nash": "wfk::nash_kernel"}[cfg.fn]
 
     result = None
     if rank == 0:
@@ -407,10 +432,9 @@ def run_ours(args, cfg):
             "e2e": {"value": total_cells / (e2e_ms * 1e-3) / 1e9, "unit": UNIT, "ms_per_step": e2e_ms,
                     "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                     "note": "H2D of the step's inputs from pinned memory, sweep, D2H of the result row"},
+            "e2e_full_grid": grid_e2e,
             "clocks": clk.summary(),
         }
-        if grid_e2e:
-            result["e2e_full_grid"] = grid_e2e
     w.close()
     if world > 1:
         dist.barrier(device_ids=[local])

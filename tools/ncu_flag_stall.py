@@ -24,12 +24,24 @@ REGIONS = {
         ("wf_nw.cuh", 756, 784, "x warp: row-code staging (polls consumer counters)"),
         ("wf_nw.cuh", 786, 834, "kernel entry / exit"),
     ],
+    "nw8": [
+        ("wf_nw8.cu", 242, 292, "compute: cell step (DPX chain, staging STS, east ring STS)"),
+        ("wf_nw8.cu", 293, 331, "compute: block (x codes, west ring LDS)"),
+        ("wf_nw8.cu", 332, 343, "compute: TMA store publish"),
+        ("wf_nw8.cu", 344, 350, "compute: block barrier (lockstep wait)"),
+        ("wf_nw8.cu", 351, 394, "compute: lag / drain barriers, run loop"),
+        ("wf_nw8.cu", 176, 241, "compute: setup"),
+        ("wf_nw8.cu", 398, 415, "helper: spin on a stale global quad (stall on flag)"),
+        ("wf_nw8.cu", 427, 559, "helper warp: global ring in/out + its barriers"),
+        ("wf_nw8.cu", 561, 611, "kernel entry / dispatch / exit"),
+    ],
     "syn": [
-        ("wf_syn.cu", 211, 222, "compute: dependency wait (wait_ctr: west hand-off / ring slot)"),
-        ("wf_syn.cu", 100, 210, "compute: cells, staging"),
-        ("wf_syn.cu", 223, 360, "compute: row blocks, TMA store, publish"),
-        ("wf_syn.cu", 365, 428, "feeder warp: west words from the LL ring (polls)"),
-        ("wf_syn.cu", 429, 483, "kernel entry / exit"),
+        ("wf_syn.cu", 236, 248, "compute: dependency wait (wait_ctr: west hand-off / ring slot)"),
+        ("wf_syn.cu", 118, 235, "compute: cells, staging, next-row word loads"),
+        ("wf_syn.cu", 249, 301, "compute: step loop (lane hand-off shuffles, east LL stores)"),
+        ("wf_syn.cu", 303, 387, "compute: block loop, TMA store, publish"),
+        ("wf_syn.cu", 397, 467, "feeder warp: west words from the LL ring (polls)"),
+        ("wf_syn.cu", 470, 535, "kernel entry / exit"),
     ],
 }
 POLL = ("dependency wait", "I/O warp", "x warp", "feeder warp")
