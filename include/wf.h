@@ -84,8 +84,12 @@ typedef struct {
   int32_t lane_cols;    /* tunable k: adjacent columns owned by one lane (1, 2, 4, 8); 0 = default */
   int32_t warps;        /* tunable: compute warps per CTA = column groups per band (1..8); 0 = default */
   int32_t skew;         /* tunable d: row lag between neighbouring lanes (1..4); 0 = default */
-  int32_t strip;        /* rows per inter-slab message of a strip transport: must be 0 (the P2P
-                           transport hands off every row; > 0 -> WF_EUNSUPPORTED) */
+  int32_t strip;        /* tunable: rows per hand-off block -- the unit in which a band passes its east
+                           column to the next band and a slab to the next slab (the paper's halo-swap
+                           interval).  0 = default (16).  Generation 8
+                           compiles 8 / 16 / 32 for its main tilings (wf_query reports the one that
+                           runs); the other generations have a fixed block and need 0; other values
+                           -> WF_EUNSUPPORTED */
   int32_t ngpus;        /* slabs (column blocks), 1..8; see wf_dist */
   int32_t match, mismatch, gap;  /* SEQCMP scores, each in [-64, 64]; defaults used if all three 0 */
   int32_t local;        /* SEQCMP: 0 = global (Needleman-Wunsch), 1 = local (Smith-Waterman) */
@@ -135,7 +139,9 @@ typedef struct {
   int32_t lane_cols, warps, skew;  /* effective tunables after defaults */
   int32_t band_cols;               /* columns per CTA band = warps * 32 * lane_cols (NASH: warps) */
   int32_t nbands;                  /* bands in this slab */
-  int32_t reserved[5];
+  int32_t strip;                   /* rows per hand-off block of the kernel that runs (generation 8);
+                                      0 = fixed by the generation */
+  int32_t reserved[4];
 } wf_layout;
 
 /* Device buffers for one wf_run.  All pointers are DEVICE pointers on the slab's device,

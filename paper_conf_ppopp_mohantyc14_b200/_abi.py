@@ -47,7 +47,7 @@ class WfLayout(ctypes.Structure):
                 ("col_begin", ctypes.c_int32), ("col_end", ctypes.c_int32), ("min_pitch", ctypes.c_int64),
                 ("bytes_out", ctypes.c_int64), ("lane_cols", ctypes.c_int32), ("warps", ctypes.c_int32),
                 ("skew", ctypes.c_int32), ("band_cols", ctypes.c_int32), ("nbands", ctypes.c_int32),
-                ("reserved", ctypes.c_int32 * 5)]
+                ("strip", ctypes.c_int32), ("reserved", ctypes.c_int32 * 4)]
 
 
 class WfIo(ctypes.Structure):

@@ -29,6 +29,7 @@ struct wf_ctx {
   int grid = 1;
   int smem = 0;
   int impl = 0;
+  int strip = 0;                           // rows per hand-off block of the variant that runs
   void* base = nullptr;                    // one allocation: [control block | edge rings] (IPC-exportable)
   unsigned* ack = nullptr;                 // control word written by the successor slab
   unsigned long long* edge = nullptr;      // nbands * rows * nf LL words (library-owned)
@@ -75,6 +76,7 @@ wf_status cuda_fail(wf_ctx* c, cudaError_t e, const char* what) {
 struct Plan {
   int nf, nbound, k, warps, skew, band_w, c0, c1, nbands;
   int impl;   // kernel generation actually used (wf_params.kernel, or the default's)
+  int strip;  // wf_params.strip (0 = the generation's default block)
   int match, mismatch, gap;
 };
 
@@ -131,14 +133,13 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   const int G = p->ngpus ? p->ngpus : 1;
   if (rank < 0 || rank >= G) return fail(c, WF_EINVAL, "rank=%d out of range for ngpus=%d", rank, G);
   if (p->transport > WF_TRANSPORT_NCCL) return fail(c, WF_EINVAL, "transport=%u unknown", p->transport);
-  // The slab hand-off is per-row P2P LL words stored by the sweep itself; the
-  // host-driven NCCL strip exchange and its strip size are not built, and are refused rather
-  // than silently ignored.
+  // The slab hand-off is P2P stores issued by the sweep itself; a host-driven
+  // NCCL exchange is not built, and is refused rather than silently ignored.
   if (p->transport == WF_TRANSPORT_NCCL)
-    return fail(c, WF_EUNSUPPORTED, "transport=NCCL is not built (P2P per-row hand-off only, DESIGN.md §8)");
-  if (p->strip < 0) return fail(c, WF_EINVAL, "strip=%d must be >= 0", p->strip);
-  if (p->strip > 0)
-    return fail(c, WF_EUNSUPPORTED, "strip=%d: the P2P transport hands off every row; strip must be 0", p->strip);
+    return fail(c, WF_EUNSUPPORTED, "transport=NCCL is not built (P2P hand-off only, DESIGN.md §8)");
+  // strip = rows per hand-off block (the band-to-band and slab-to-slab message); selectable
+  // for generation 8 among its compiled blocks, fixed (0) for the other generations
+  if (p->strip < 0 || p->strip > 65535) return fail(c, WF_EINVAL, "strip=%d out of range 0..65535", p->strip);
   if (p->lane_cols < 0 || p->warps < 0 || p->skew < 0)
     return fail(c, WF_EINVAL, "lane_cols/warps/skew must be >= 0");
   Plan pl{};
@@ -176,16 +177,21 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
       return fail(c, WF_EINVAL, "fn=%d unknown", p->fn);
   }
   defaults(*p, &pl.k, &pl.warps, &pl.skew, &pl.impl);
+  pl.strip = p->strip;
   if (pl.k != 1 && pl.k != 2 && pl.k != 4 && pl.k != 8) return fail(c, WF_EINVAL, "lane_cols=%d not in {1,2,4,8}", pl.k);
   if (pl.warps < 1 || pl.warps > 8) return fail(c, WF_EINVAL, "warps=%d out of range 1..8", pl.warps);
   if (pl.skew < 1 || pl.skew > 4) return fail(c, WF_EINVAL, "skew=%d out of range 1..4", pl.skew);
   // a default band width whose shared-memory rings do not fit (many planes) halves until it does
   while (!p->warps && pl.warps > 1 &&
-         !wfk::variant_exists(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew, pl.impl))
+         !wfk::variant_exists(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew, pl.impl,
+                              pl.strip))
     pl.warps /= 2;
-  if (!wfk::variant_exists(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew, pl.impl))
-    return fail(c, WF_EUNSUPPORTED, "no kernel variant for fn=%d dsize=%d lane_cols=%d warps=%d skew=%d", p->fn,
-                p->dsize, pl.k, pl.warps, pl.skew);
+  if (!wfk::variant_exists(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew, pl.impl,
+                           pl.strip))
+    return fail(c, WF_EUNSUPPORTED, "no kernel variant for fn=%d dsize=%d lane_cols=%d warps=%d skew=%d strip=%d",
+                p->fn, p->dsize, pl.k, pl.warps, pl.skew, pl.strip);
+  pl.strip = wfk::variant_strip(p->fn, p->fn == WF_FN_SEQCMP ? p->local : p->dsize, pl.k, pl.warps, pl.skew, pl.impl,
+                                pl.strip);
   pl.band_w = p->fn == WF_FN_NASH ? pl.warps : pl.warps * 32 * pl.k;   // NASH: one column per warp
   // slabs: every slab but the last is a whole number of bands (its east column is then
   // owned by the last lane of its last band); bands are dealt out as evenly as possible
@@ -242,6 +248,7 @@ wf_status wf_query(const wf_params* p, int32_t rank, wf_layout* out) {
   out->skew = pl.skew;
   out->band_cols = pl.band_w;
   out->nbands = pl.nbands;
+  out->strip = pl.strip;
   return WF_OK;
 }
 
@@ -274,6 +281,7 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   c->k = pl.k;
   c->warps = pl.warps;
   c->impl = pl.impl;
+  c->strip = pl.strip;
   c->skew = pl.skew;
   c->band_w = pl.band_w;
   c->nbands = pl.nbands;
@@ -302,6 +310,7 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   L.dsize = p->dsize;
   L.local = p->fn == WF_FN_SEQCMP ? p->local : 0;
   L.impl = pl.impl;
+  L.strip = pl.strip;
   L.k = pl.k;
   L.warps = pl.warps;
   L.skew = pl.skew;
@@ -406,7 +415,7 @@ wf_status wf_link_local(wf_ctx* prev, wf_ctx* next) {
   if (prev->nf != next->nf || prev->p.dim != next->p.dim || prev->p.fn != next->p.fn ||
       prev->p.cols != next->p.cols || prev->p.tsize != next->p.tsize || prev->p.dsize != next->p.dsize ||
       prev->p.local != next->p.local || prev->impl != next->impl || prev->k != next->k ||
-      prev->warps != next->warps || prev->skew != next->skew)
+      prev->warps != next->warps || prev->skew != next->skew || prev->strip != next->strip)
     return fail(prev, WF_EINVAL, "wf_link_local: contexts describe different problems or tunings");
   if (prev->c1 != next->c0)
     return fail(prev, WF_EINVAL, "wf_link_local: slab %d ends at column %d but slab %d starts at %d", prev->rank,
@@ -535,6 +544,7 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   L.dsize = p.dsize;
   L.local = p.fn == WF_FN_SEQCMP ? p.local : 0;
   L.impl = c->impl;
+  L.strip = c->strip;
   L.lane_best = c->lane_best;
   L.best_out = c->best_out;
   L.c0 = c->c0;

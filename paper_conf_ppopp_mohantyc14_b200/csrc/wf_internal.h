@@ -46,7 +46,8 @@ struct SweepLaunch {
   // [nbands][warps][32]; the slab's best cell (value, 1-based row, 1-based global column)
   int32_t local;
   int32_t cluster;
-  int32_t impl;        // wf_params.kernel: 0 default, 4 first generation, 7 second generation     // SEQCMP v4: launched as clusters of 8 CTAs, band-to-band hand-off via DSMEM
+  int32_t impl;        // wf_params.kernel actually used (0 = the function's default generation)
+  int32_t strip;       // wf_params.strip: rows per hand-off block (generation 8); 0 = the default
   int2* lane_best;
   int32_t* best_out;
 };
@@ -66,7 +67,9 @@ cudaError_t launch(const SweepLaunch& L, cudaStream_t s);
 // Finish the Smith-Waterman best-cell reduction of a run (after the sweep, same stream).
 cudaError_t launch_sw_best(const SweepLaunch& L, cudaStream_t s);
 // Is (fn, dsize, k, warps, skew) compiled?  (SEQCMP: dsize carries the local flag.)
-bool variant_exists(int fn, int dsize, int k, int warps, int skew, int impl = 0);
+bool variant_exists(int fn, int dsize, int k, int warps, int skew, int impl = 0, int strip = 0);
+// Rows per hand-off block of the variant that runs (generation 8: its U; 0 for the others).
+int variant_strip(int fn, int dsize, int k, int warps, int skew, int impl, int strip);
 
 constexpr int kTraceSlots = 64;   // per band: [0..32] row stamps, [40] feeder polls, [41] empty polls,
 constexpr int kTraceRows = 32;    // [42] last warp's first outbound stamp

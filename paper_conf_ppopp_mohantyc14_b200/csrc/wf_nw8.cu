@@ -64,7 +64,7 @@ namespace nw8 {
 #define WF_NW8_DPRE 1  // blocks ahead the helper loads the inbound words (A/B 1 / 2 / 3: 1.96 / 2.02 / 2.06 ms)
 #endif
 
-constexpr int RR = 64;         // slots per shared ring (power of 2, > 2U)
+constexpr int RR = 128;        // slots per shared ring (power of 2, > 2U for every compiled U <= 32)
 constexpr int SR = 128;        // staging rows per warp (power of 2, = 4 TMA boxes)
 constexpr int XPAD = 64;       // bytes of padding around the shared x copy
 constexpr int XMAX = 65536;    // rows the shared x copy holds (ABI maximum 65535)
@@ -612,33 +612,39 @@ __global__ void __launch_bounds__((WARPS + 1) * 32, 1)
 
 constexpr int kU = WF_NW8_U;   // steps per lockstep block
 
-template <int K, int WARPS>
+template <int K, int WARPS, int U>
 cudaError_t launch(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   CUtensorMap tmap;
   cudaError_t e = encode_plane_map(&tmap, L, 32 * K, 32);
   if (e != cudaSuccess) return e;
-  auto kfn = L.local ? nw8_kernel<K, WARPS, true, kU> : nw8_kernel<K, WARPS, false, kU>;
+  auto kfn = L.local ? nw8_kernel<K, WARPS, true, U> : nw8_kernel<K, WARPS, false, U>;
   e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
   kfn<<<L.grid, (WARPS + 1) * 32, smem, s>>>(L, tmap);
   return cudaGetLastError();
 }
 
-template <int K, int WARPS, bool LOCAL>
+// U = the strip (wf_params.strip): rows per lockstep block, per band-to-band / slab-to-slab
+// hand-off and per helper message
+template <int K, int WARPS, bool LOCAL, int U = kU>
 Variant make() {
   return Variant{WF_FN_SEQCMP, LOCAL ? 1 : 0, K, WARPS, 1, (WARPS + 1) * 32, Smem<K, WARPS>::bytes,
-                 reinterpret_cast<const void*>(nw8_kernel<K, WARPS, LOCAL, kU>), &launch<K, WARPS>, 8, {}};
+                 reinterpret_cast<const void*>(nw8_kernel<K, WARPS, LOCAL, U>), &launch<K, WARPS, U>, 8, {}, U};
 }
 
 }  // namespace nw8
 
 // Both the global (local = 0) and the Smith-Waterman (local = 1, looked up with dsize = 1)
-// variants; each entry's kernel pointer is the exact instantiation launch() uses.
+// variants; each entry's kernel pointer is the exact instantiation launch() uses.  The first
+// entry of a (K, warps, local) is its default strip (kU); the strip axis (8 / 32 rows) is
+// compiled for the two main tilings.
 const Variant* nw8_table(size_t* n) {
   static const Variant v[] = {
-      nw8::make<2, 4, false>(), nw8::make<2, 2, false>(), nw8::make<1, 4, false>(), nw8::make<1, 8, false>(),
-      nw8::make<4, 2, false>(), nw8::make<4, 1, false>(), nw8::make<2, 1, false>(), nw8::make<2, 4, true>(),
-      nw8::make<2, 2, true>(),  nw8::make<1, 4, true>(),  nw8::make<4, 2, true>(),
+      nw8::make<2, 4, false>(),     nw8::make<2, 2, false>(),     nw8::make<1, 4, false>(),
+      nw8::make<1, 8, false>(),     nw8::make<4, 2, false>(),     nw8::make<4, 1, false>(),
+      nw8::make<2, 1, false>(),     nw8::make<2, 4, true>(),      nw8::make<2, 2, true>(),
+      nw8::make<1, 4, true>(),      nw8::make<4, 2, true>(),      nw8::make<2, 4, false, 8>(),
+      nw8::make<2, 4, false, 32>(), nw8::make<4, 2, false, 8>(),  nw8::make<4, 2, false, 32>(),
   };
   *n = sizeof(v) / sizeof(v[0]);
   return v;

@@ -183,16 +183,19 @@ const Variant* table(size_t* n) {
   return v;
 }
 
-const Variant* find(int fn, int dsize, int k, int warps, int skew, int impl) {
+const Variant* find(int fn, int dsize, int k, int warps, int skew, int impl, int strip) {
   size_t n;
-  // SEQCMP: generation 8 (the default, wf_nw8.cu) for its compiled (K, warps) at skew 1; every
-  // other tuning -- or kernel = 4 -- runs generation 4 (wf_nw.cuh, wf_sw.cu)
+  // SEQCMP: generation 8 (the default, wf_nw8.cu) for its compiled (K, warps, strip) at skew 1;
+  // every other tuning -- or kernel = 4 -- runs generation 4 (wf_nw.cuh, wf_sw.cu).  strip 0 =
+  // generation 8's default block (the first entry of a (K, warps) in its table).
   if (fn == WF_FN_SEQCMP && skew == 1 && (impl == 0 || impl == 8)) {
     const Variant* t8 = nw8_table(&n);
     for (size_t i = 0; i < n; ++i)
-      if (t8[i].dsize == dsize && t8[i].k == k && t8[i].warps == warps) return &t8[i];
-    if (impl == 8) return nullptr;
+      if (t8[i].dsize == dsize && t8[i].k == k && t8[i].warps == warps && (strip == 0 || t8[i].strip == strip))
+        return &t8[i];
+    if (impl == 8 || strip != 0) return nullptr;
   }
+  if (strip != 0) return nullptr;   // the other generations' blocks are fixed
   if (fn == WF_FN_SEQCMP && dsize == 1) {   // local alignment (Smith-Waterman)
     const Variant* ts = sw_table(&n);
     for (size_t i = 0; i < n; ++i)
@@ -220,21 +223,26 @@ const Variant* find(int fn, int dsize, int k, int warps, int skew, int impl) {
 
 }  // namespace
 
-bool variant_exists(int fn, int dsize, int k, int warps, int skew, int impl) {
+bool variant_exists(int fn, int dsize, int k, int warps, int skew, int impl, int strip) {
   // compiled AND within the 227 KB per-CTA shared-memory limit of sm_100
-  const Variant* v = find(fn, (fn == WF_FN_SYNTHETIC || fn == WF_FN_SEQCMP) ? dsize : 0, k, warps, skew, impl);
+  const Variant* v = find(fn, (fn == WF_FN_SYNTHETIC || fn == WF_FN_SEQCMP) ? dsize : 0, k, warps, skew, impl, strip);
   return v != nullptr && v->smem <= 232448;
 }
 
+int variant_strip(int fn, int dsize, int k, int warps, int skew, int impl, int strip) {
+  const Variant* v = find(fn, (fn == WF_FN_SYNTHETIC || fn == WF_FN_SEQCMP) ? dsize : 0, k, warps, skew, impl, strip);
+  return v ? v->strip : 0;
+}
+
 int smem_bytes(const SweepLaunch& L) {
-  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew, L.impl);
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew, L.impl, L.strip);
   if (!v) return -1;
   if (L.fn == WF_FN_NASH) return (int)(v->smem + size_t(L.warps) * ((size_t(2) * L.tsize * L.tsize + 2 * L.tsize + 15) & ~size_t(15)));
   return (int)v->smem;
 }
 
 int occupancy(const SweepLaunch& L, int smem) {
-  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew, L.impl);
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew, L.impl, L.strip);
   if (!v) return 0;
   if (cudaFuncSetAttribute(v->kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem) != cudaSuccess) {
     cudaGetLastError();
@@ -261,7 +269,7 @@ int occupancy(const SweepLaunch& L, int smem) {
 }
 
 cudaError_t launch(const SweepLaunch& L, cudaStream_t s) {
-  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew, L.impl);
+  const Variant* v = find(L.fn, L.fn == WF_FN_SYNTHETIC ? L.dsize : (L.fn == WF_FN_SEQCMP ? L.local : 0), L.k, L.warps, L.skew, L.impl, L.strip);
   if (!v) return cudaErrorInvalidDeviceFunction;
   return v->launch(L, s, (size_t)smem_bytes(L));
 }

@@ -16,6 +16,8 @@ struct Variant {
   int impl;            // kernel generation (SEQCMP: 4 = block hand-offs, 8 = lane pipeline)
   const void* alt[4];  // other instantiations launch() may pick for this variant (e.g. compile-time
                        // tsize); occupancy() takes the minimum over kernel and alt[]
+  int strip;           // rows per hand-off block = rows per inter-slab message (generation 8: U);
+                       // 0 = fixed by the generation (not selectable)
 };
 
 // SEQCMP v8 variants (wf_nw8.cu): global (dsize 0) and local / Smith-Waterman (dsize 1)

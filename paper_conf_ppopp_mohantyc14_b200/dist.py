@@ -30,6 +30,44 @@ def neighbour_handles(my_handle: bytes, rank: int, world: int, group=None) -> tu
     return prev, nxt
 
 
+def slab_fingerprint(w) -> tuple:
+    """What every rank must agree on before wf_connect: the problem and the tuning (equal on all
+    ranks) and this slab's column range (consecutive across ranks).  wf_link_local checks the same
+    in C for slabs of one process; across processes the IPC handle carries only memory."""
+    p, lay = w.params, w.layout
+    problem = (int(p.fn), int(p.dim), int(p.cols), int(p.tsize), int(p.dsize), int(p.local), int(p.match),
+               int(p.mismatch), int(p.gap), int(p.alphabet), int(p.ngpus))
+    tuning = (int(lay.lane_cols), int(lay.warps), int(lay.skew), int(lay.strip), int(p.kernel))
+    return problem, tuning, (int(lay.col_begin), int(lay.col_end))
+
+
+def check_fingerprints(fps: list) -> None:
+    """Raise ValueError unless all ranks describe the same problem and tuning and their slabs are
+    consecutive column blocks covering [0, cols)."""
+    for g, (prob, tun, _) in enumerate(fps):
+        if prob != fps[0][0]:
+            raise ValueError(f"rank {g} describes a different problem than rank 0: {prob} vs {fps[0][0]}")
+        if tun != fps[0][1]:
+            raise ValueError(f"rank {g} uses a different tuning than rank 0: {tun} vs {fps[0][1]}")
+    if fps[0][2][0] != 0:
+        raise ValueError(f"rank 0 starts at column {fps[0][2][0]}")
+    for g in range(1, len(fps)):
+        if fps[g][2][0] != fps[g - 1][2][1]:
+            raise ValueError(f"slab {g - 1} ends at column {fps[g - 1][2][1]} but slab {g} starts at {fps[g][2][0]}")
+
+
+def exchange_handles(my_handle: bytes, fingerprint: tuple, rank: int, world: int,
+                     group=None) -> tuple[bytes | None, bytes | None]:
+    """All-gather (handle, fingerprint) of every rank, validate the fingerprints
+    (check_fingerprints, identical verdict on every rank), return (handle of rank-1, of rank+1)."""
+    recs: list = [None] * world
+    dist.all_gather_object(recs, (bytes(my_handle), fingerprint), group=group)
+    check_fingerprints([r[1] for r in recs])
+    prev = recs[rank - 1][0] if rank > 0 else None
+    nxt = recs[rank + 1][0] if rank < world - 1 else None
+    return prev, nxt
+
+
 def max_over_ranks(x: float, device=None, group=None) -> float:
     """Max of a per-rank time (ms) over all ranks (BASELINE timing rule: max over ranks)."""
     t = torch.tensor([float(x)], dtype=torch.float64, device=device)
@@ -38,6 +76,7 @@ def max_over_ranks(x: float, device=None, group=None) -> float:
 
 
 def connect_slab(w, rank: int, world: int, group=None) -> None:
-    """Link a rank's Wavefront context to its neighbours' edge rings (wf_connect)."""
-    prev, nxt = neighbour_handles(w.ipc_handle(), rank, world, group)
+    """Link a rank's Wavefront context to its neighbours' edge rings (wf_connect), after checking
+    that all ranks agree on problem, tuning and slab adjacency (ValueError otherwise)."""
+    prev, nxt = exchange_handles(w.ipc_handle(), slab_fingerprint(w), rank, world, group)
     w.connect(prev, nxt)

@@ -32,6 +32,7 @@ class Layout:
     skew: int
     band_cols: int
     nbands: int
+    strip: int = 0   # rows per hand-off block (generation 8); 0 = fixed by the generation
 
     @property
     def width(self) -> int:
@@ -68,7 +69,7 @@ def query(fn, dim, rank: int = 0, **kw) -> Layout:
     check(_abi.lib().wf_query(ctypes.byref(p), int(rank), ctypes.byref(lay)))
     return Layout(lay.nplanes, [bool(lay.plane_is_float[i]) for i in range(lay.nplanes)], lay.nbound,
                   lay.col_begin, lay.col_end, lay.min_pitch, lay.bytes_out, lay.lane_cols, lay.warps,
-                  lay.skew, lay.band_cols, lay.nbands)
+                  lay.skew, lay.band_cols, lay.nbands, lay.strip)
 
 
 def _stream_handle(stream) -> int:

@@ -68,12 +68,29 @@ def test_query_rejects_bad_params_naming_the_field(kw, field):
     assert field in str(e)
 
 
-@pytest.mark.parametrize("kw,field", [(dict(transport="nccl"), "transport"), (dict(strip=256), "strip")])
-def test_unbuilt_transport_options_are_refused(kw, field):
-    # the slab hand-off is the sweep's own per-row P2P store; the NCCL strip
-    # transport is not built and must not be accepted and silently ignored
-    e = _err("seqcmp", 256, ngpus=2, **kw)
-    assert e.status == _abi.WF_EUNSUPPORTED and field in str(e)
+def test_unbuilt_nccl_transport_is_refused():
+    # the slab hand-off is the sweep's own P2P store; an NCCL transport is not
+    # built and must not be accepted and silently ignored
+    e = _err("seqcmp", 256, ngpus=2, transport="nccl")
+    assert e.status == _abi.WF_EUNSUPPORTED and "transport" in str(e)
+
+
+def test_strip_axis():
+    """wf_params.strip = rows per hand-off block: generation 8 compiles 8 / 16 / 32 for its main
+    tilings (default 16, reported by wf_query); other strips, and any strip on a generation with a
+    fixed block, are refused by name."""
+    assert query("seqcmp", 1000).strip == 16
+    for s in (8, 16, 32):
+        assert query("seqcmp", 1000, lane_cols=2, warps=4, strip=s).strip == s
+        assert query("seqcmp", 1000, lane_cols=4, warps=2, strip=s, ngpus=2).strip == s
+    assert query("seqcmp", 1000, lane_cols=1, warps=4).strip == 16
+    for kw in (dict(strip=24), dict(strip=8, lane_cols=1, warps=4), dict(strip=16, kernel=4),
+               dict(strip=16, skew=2, lane_cols=4, warps=1)):
+        e = _err("seqcmp", 1000, **kw)
+        assert e.status == _abi.WF_EUNSUPPORTED and "strip" in str(e)
+    assert query("synthetic", 100, tsize=10, dsize=1).strip == 0
+    assert _err("synthetic", 100, tsize=10, dsize=1, strip=16).status == _abi.WF_EUNSUPPORTED
+    assert _err("seqcmp", 1000, strip=-1).status == _abi.WF_EINVAL
 
 
 def test_reserved_fields_must_be_zero():

@@ -35,6 +35,17 @@ def test_link_rejects_a_different_tuning():
         b.close()
 
 
+def test_link_rejects_a_different_strip():
+    a, b = _slab(0, strip=8), _slab(1, strip=32)
+    try:
+        with pytest.raises(_abi.WfError) as ei:
+            a.link(b)
+        assert ei.value.status == _abi.WF_EINVAL
+    finally:
+        a.close()
+        b.close()
+
+
 def test_link_rejects_non_adjacent_slabs():
     a, c = _slab(0, G=3, dim=1000), _slab(2, G=3, dim=1000)
     try:

@@ -39,6 +39,21 @@ def _worker(rank, world, port, q):
             res[(fn, dim)] = allb
         prev, nxt = wdist.neighbour_handles(f"handle-of-rank-{rank}".encode(), rank, world)
         res["handles"] = (prev, nxt)
+        # connect-time validation: the same problem / tuning on every rank, consecutive slabs
+        prob = (2, 1000, 0, 0, 0, 0, 1, -1, -1, 0, world)
+        bounds = wdist.slab_bounds("seqcmp", 1000, rank, world)
+        ok = wdist.exchange_handles(b"h%d" % rank, (prob, (2, 4, 1, 16, 0), bounds), rank, world)
+        res["fp_ok"] = ok
+        verdicts = []
+        for bad in ("strip", "bounds"):
+            tun = (2, 4, 1, 32 if (bad == "strip" and rank == 1) else 16, 0)
+            b = (bounds[0] + (1 if bad == "bounds" and rank == 1 else 0), bounds[1])
+            try:
+                wdist.exchange_handles(b"h%d" % rank, (prob, tun, b), rank, world)
+                verdicts.append("accepted")
+            except ValueError as e:
+                verdicts.append(str(e)[:40])
+        res["fp_bad"] = verdicts
         res["max"] = wdist.max_over_ranks(1.5 * rank + 0.25)
         q.put((rank, res))
     finally:
@@ -68,3 +83,19 @@ def test_two_rank_slab_partition_handles_and_max(world):
         assert prev == (None if rank == 0 else f"handle-of-rank-{rank - 1}".encode())
         assert nxt == (None if rank == world - 1 else f"handle-of-rank-{rank + 1}".encode())
         assert r["max"] == 1.5 * (world - 1) + 0.25
+        assert r["fp_ok"] == ((None if rank == 0 else b"h%d" % (rank - 1)), (None if rank == world - 1 else b"h%d" % (rank + 1)))
+        # every rank refuses (the same verdict on both sides of the link)
+        assert r["fp_bad"][0].startswith("rank 1 uses a different tuning")
+        assert r["fp_bad"][1].startswith("slab 0 ends at column")
+
+
+def test_check_fingerprints_single_process():
+    from paper_conf_ppopp_mohantyc14_b200.dist import check_fingerprints
+    prob, tun = (2, 100, 0, 0, 0, 0, 1, -1, -1, 0, 3), (2, 4, 1, 16, 0)
+    check_fingerprints([(prob, tun, (0, 40)), (prob, tun, (40, 80)), (prob, tun, (80, 100))])
+    for fps, msg in (([(prob, tun, (0, 40)), (prob[:1] + (101,) + prob[2:], tun, (40, 100))], "problem"),
+                     ([(prob, tun, (0, 40)), (prob, (2, 4, 1, 8, 0), (40, 100))], "tuning"),
+                     ([(prob, tun, (0, 40)), (prob, tun, (50, 100))], "ends at column"),
+                     ([(prob, tun, (5, 40)), (prob, tun, (40, 100))], "starts at column")):
+        with pytest.raises(ValueError, match=msg):
+            check_fingerprints(fps)

@@ -106,6 +106,37 @@ def test_nw_brute_force_all_prefixes(scoring):
                 assert H[i - 1, j - 1] == max(_all_global_alignment_scores(x[:i], y[:j], M, X, G))
 
 
+@pytest.mark.parametrize("kind", ["protein", "bytes"])
+def test_nw_brute_force_any_byte_residues(kind):
+    """alphabet = 0 inputs (ASCII letters, bytes >= 0x80): the oracle still equals the maximum
+    over all alignments -- only equality of codes enters s(x_i, y_j)."""
+    M, X, G = 2, -1, -1
+    for t in range(8):
+        x, y = workloads.seqcmp_inputs(int(3 + t % 4), int(6 - t % 3), kind=kind, seed_x=40 + t, seed_y=80 + t)
+        if t % 2:   # force some matches
+            y[: min(len(x), len(y)) // 2] = x[: min(len(x), len(y)) // 2]
+        H = oracle.seqcmp(x, y, M, X, G)
+        for i in range(1, len(x) + 1):
+            for j in range(1, len(y) + 1):
+                assert H[i - 1, j - 1] == max(_all_global_alignment_scores(x[:i], y[:j], M, X, G))
+
+
+def test_nw_invariant_under_residue_relabelling():
+    """A bijection of the byte alphabet leaves the grid unchanged (s depends on x_i == y_j only);
+    0x80..0xff codes behave like any other (no sign-extension artefacts)."""
+    x, y = workloads.seqcmp_inputs(200, 230, kind="bytes")
+    perm = np.random.default_rng(5).permutation(256).astype(np.uint8)
+    for local in (False, True):
+        H = oracle.seqcmp(x, y, 2, -1, -1, local=local)
+        assert np.array_equal(H, oracle.seqcmp(perm[x], perm[y], 2, -1, -1, local=local))
+    px, py = workloads.seqcmp_inputs(150, kind="protein")
+    assert set(np.unique(px)) <= set(workloads.PROTEIN) and len(np.unique(px)) == 20
+    codes = {c: i for i, c in enumerate(workloads.PROTEIN)}
+    assert np.array_equal(oracle.seqcmp(px, py, 1, -1, -1),
+                          oracle.seqcmp(np.array([codes[c] for c in px], np.uint8),
+                                        np.array([codes[c] for c in py], np.uint8), 1, -1, -1))
+
+
 def test_sw_local_brute_force():
     """Smith-Waterman H[i][j] == max(0, best alignment of a suffix of x[:i] with a suffix of y[:j])."""
     M, X, G = 2, -1, -1

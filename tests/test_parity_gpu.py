@@ -67,6 +67,22 @@ def test_seqcmp_generation8_variants(k, w, dim):
     assert np.array_equal(H, g)
 
 
+@pytest.mark.parametrize("k,w", [(2, 4), (4, 2)])
+@pytest.mark.parametrize("strip", [8, 32])
+@pytest.mark.parametrize("dim", [1, 33, 97, 777, 3001])
+def test_seqcmp_generation8_strips(k, w, strip, dim):
+    """wf_params.strip: rows per hand-off block (8 / 32 besides the default 16)."""
+    H, g = _seq(dim, lane_cols=k, warps=w, skew=1, kernel=8, strip=strip, seed=(dim + 1, dim + 2))
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.parametrize("strip", [8, 32])
+@pytest.mark.parametrize("G", [2, 3])
+def test_seqcmp_strips_local_slabs(strip, G):
+    H, g = _seq(1000, ngpus=G, strip=strip, seed=(5, 6))
+    assert np.array_equal(H, g)
+
+
 @pytest.mark.parametrize("k,w,d", [(4, 2, 1), (2, 4, 1), (4, 1, 2)])
 @pytest.mark.parametrize("dim", [33, 777, 1100])
 def test_seqcmp_generation4_kernel(k, w, d, dim):
@@ -165,6 +181,35 @@ def test_seqcmp_byte_permute_scores(alphabet, scoring):
 @pytest.mark.parametrize("scoring", [(1, -1, -1), (1, -1, -2), (2, -3, -1), (5, -4, -10), (64, -64, -64), (0, 0, 1)])
 def test_seqcmp_input_kinds_and_scorings(kind, scoring):
     H, g = _seq(613, kind=kind, scoring=scoring)
+    assert np.array_equal(H, g)
+
+
+ASCII_KINDS = ["protein", "dna_ascii", "bytes"]
+
+
+@pytest.mark.parametrize("kind", ASCII_KINDS)
+@pytest.mark.parametrize("k,w,d,kernel", [(2, 4, 1, 8), (4, 2, 1, 8), (1, 4, 1, 8), (2, 1, 1, 8), (4, 2, 1, 4),
+                                          (4, 1, 2, 4), (8, 1, 1, 4)])
+def test_seqcmp_any_byte_residues(kind, k, w, d, kernel):
+    """alphabet = 0 (include/wf.h: codes may be any byte value): ASCII amino-acid and DNA
+    letters, and raw bytes 0..255 (codes >= 0x80 must not sign-extend into a false match)."""
+    for dim, cols, scoring in ((1100, 0, (2, -1, -1)), (777, 1301, (5, -4, -10))):
+        H, g = _seq(dim, cols=cols, kind=kind, scoring=scoring, seed=(dim + 3, cols + 5), lane_cols=k, warps=w, skew=d,
+                    kernel=kernel, alphabet=0)
+        assert np.array_equal(H, g), (kind, dim, cols)
+
+
+@pytest.mark.parametrize("kind", ASCII_KINDS)
+def test_smith_waterman_any_byte_residues(kind):
+    for k, w, d in ((2, 4, 1), (4, 2, 1), (4, 1, 2)):
+        H, g, best = _sw_run(1000, cols=1200, kind=kind, scoring=(2, -1, -1), lane_cols=k, warps=w, skew=d, alphabet=0)
+        assert np.array_equal(H, g)
+        assert best == _sw_expect(H)
+
+
+@pytest.mark.parametrize("G", [2, 3])
+def test_seqcmp_any_byte_residues_local_slabs(G):
+    H, g = _seq(1000, kind="bytes", ngpus=G, alphabet=0)
     assert np.array_equal(H, g)
 
 

@@ -8,9 +8,10 @@ paper's ML-tuned parameters"; Table 2, P:395-422 S
 The paper's tunables (cpu-tile, band, gpu-count, gpu-tile, halo) map onto this build's
 (DESIGN.md §6-7):
   * tile      -> lane_cols K (columns per lane) x warps W (the CTA band is 32*K*W columns),
-  * strip     -> lane skew D (rows between neighbouring lanes) and, for sequence comparison,
-                 the kernel generation (wf_params.kernel 8 = lockstep lane pipeline, 4 = U-row
-                 block hand-offs),
+  * strip     -> wf_params.strip S: rows per hand-off block, i.e. per band-to-band and
+                 slab-to-slab message (generation 8: 8 / 16 / 32), plus the lane skew D and the
+                 kernel generation (wf_params.kernel 8 = lockstep lane pipeline, 4 = U-row block
+                 hand-offs),
   * gpu-count -> column slabs (--slabs G...): G slabs linked by the per-row P2P hand-off.  On one
                  physical GPU they are virtual slabs sharing its SMs (device_share) -- a
                  correctness and hand-off-cost point, not a speed-up; with G visible GPUs each slab
@@ -44,9 +45,9 @@ from paper_conf_ppopp_mohantyc14_b200.wf import LocalSlabs, Wavefront, query  # 
 # SYNTHETIC 7 = wf_syn, 4 = generic sweep, 8 = plane-split wf_syn (dsize >= 2, k = w = d = 1);
 # Nash has one kernel (0).  Combinations a generation does not compile are skipped (wf_query).
 SEARCH = {
-    "seqcmp": {"k": [1, 2, 4, 8], "w": [1, 2, 4, 8], "d": [1, 2], "impl": [8, 4]},
-    "synthetic": {"k": [1, 2], "w": [1, 2, 4], "d": [1, 2], "impl": [7, 4, 8]},
-    "nash": {"k": [1], "w": [1, 2, 4, 8], "d": [1], "impl": [0]},
+    "seqcmp": {"k": [1, 2, 4, 8], "w": [1, 2, 4, 8], "d": [1, 2], "impl": [8, 4], "s": [0, 8, 32]},
+    "synthetic": {"k": [1, 2], "w": [1, 2, 4], "d": [1, 2], "impl": [7, 4, 8], "s": [0]},
+    "nash": {"k": [1], "w": [1, 2, 4, 8], "d": [1], "impl": [0], "s": [0]},
 }
 
 
@@ -87,11 +88,11 @@ def fn_kw(cfg):
     return dict(tsize=cfg.tsize, dsize=4)
 
 
-def parity_ok(cfg, k, w, d, impl, dev, small):
+def parity_ok(cfg, k, w, d, impl, dev, small, strip=0):
     host, devin = inputs_for(cfg.fn, small, cfg.dsize, dev)
     small_cfg = workloads.Config(cfg.name, cfg.fn, small, tsize=cfg.tsize, dsize=cfg.dsize)
     want = oracle_grid(cfg.fn, host, small_cfg)
-    with Wavefront(cfg.fn, small, lane_cols=k, warps=w, skew=d, kernel=impl, **fn_kw(cfg)) as wf:
+    with Wavefront(cfg.fn, small, lane_cols=k, warps=w, skew=d, kernel=impl, strip=strip, **fn_kw(cfg)) as wf:
         out = wf.run(*devin)
         wf.sync()
         got = [o.cpu().numpy() for o in out]
@@ -108,8 +109,8 @@ def parity_ok(cfg, k, w, d, impl, dev, small):
     return True
 
 
-def time_point(cfg, k, w, d, impl, devin, reps):
-    with Wavefront(cfg.fn, cfg.dim, lane_cols=k, warps=w, skew=d, kernel=impl, **fn_kw(cfg)) as wf:
+def time_point(cfg, k, w, d, impl, devin, reps, strip=0):
+    with Wavefront(cfg.fn, cfg.dim, lane_cols=k, warps=w, skew=d, kernel=impl, strip=strip, **fn_kw(cfg)) as wf:
         out = wf.alloc_out()
         for _ in range(3):
             wf.run(*devin, out=out)
@@ -126,20 +127,25 @@ def time_point(cfg, k, w, d, impl, devin, reps):
         return statistics.median(ms), wf.layout.nbands
 
 
-def compiled(cfg, k, w, d, impl):
-    """Does the library build this (fn, tuning, generation)?  (host-side wf_query; no GPU work)"""
+def compiled(cfg, k, w, d, impl, strip=0):
+    """Does the library build this (fn, tuning, generation, strip)?  (host-side wf_query; no GPU work)"""
     try:
-        lay = query(cfg.fn, cfg.dim, lane_cols=k, warps=w, skew=d, kernel=impl, **fn_kw(cfg))
+        lay = query(cfg.fn, cfg.dim, lane_cols=k, warps=w, skew=d, kernel=impl, strip=strip, **fn_kw(cfg))
     except Exception:  # noqa: BLE001 -- WF_EUNSUPPORTED / WF_EINVAL
         return False
     return (lay.lane_cols, lay.warps, lay.skew) == (k, w, d)
 
 
-def time_slabs(cfg, k, w, d, impl, host, G, reps):
-    """G column slabs of the same grid linked by the per-row P2P hand-off (virtual slabs on one GPU)."""
+def time_slabs(cfg, k, w, d, impl, host, G, reps, strip=0):
+    """G column slabs of the same grid linked by the per-row P2P hand-off.  Virtual slabs (one
+    GPU): device time between two events on the current stream, which gates every slab stream --
+    a ~2 ms device-side sleep ahead of the start event holds the slabs back until the host has
+    enqueued all G launches, so host launch latency is not timed.  One GPU per slab: wall clock."""
     ngpu = torch.cuda.device_count()
     devices = [g % ngpu for g in range(G)]
-    ls = LocalSlabs(cfg.fn, cfg.dim, G, devices=devices, lane_cols=k, warps=w, skew=d, kernel=impl, **fn_kw(cfg))
+    ls = LocalSlabs(cfg.fn, cfg.dim, G, devices=devices, lane_cols=k, warps=w, skew=d, kernel=impl, strip=strip,
+                    **fn_kw(cfg))
+    virtual = len(set(devices)) == 1
     try:
         per = [inputs_for(cfg.fn, cfg.dim, cfg.dsize, torch.device("cuda", s.device))[1] for s in ls.slabs]
         outs = None
@@ -150,29 +156,115 @@ def time_slabs(cfg, k, w, d, impl, host, G, reps):
         for _ in range(reps):
             for dv in set(devices):
                 torch.cuda.synchronize(dv)
-            t0 = time.perf_counter()
-            outs = ls.run(per, outs)
-            ls.sync()
-            ms.append((time.perf_counter() - t0) * 1e3)
+            if virtual:
+                cur = torch.cuda.current_stream()
+                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                torch.cuda._sleep(4_000_000)
+                e0.record(cur)
+                outs = ls.run(per, outs)   # every slab stream waits on cur (LocalSlabs.run)
+                for st in ls.streams:
+                    cur.wait_stream(st)
+                e1.record(cur)
+                ls.sync()
+                torch.cuda.synchronize()
+                ms.append(e0.elapsed_time(e1))
+            else:
+                t0 = time.perf_counter()
+                outs = ls.run(per, outs)
+                ls.sync()
+                ms.append((time.perf_counter() - t0) * 1e3)
         return statistics.median(ms)
     finally:
         ls.close()
 
 
+# tunings tried per G on the gpu-count axis (the config default is always tried first)
+SLAB_TUNINGS = {   # (lane_cols, warps, skew, kernel, strip)
+    "seqcmp": [(2, 4, 1, 8, 8), (2, 4, 1, 8, 32), (4, 2, 1, 8, 0), (2, 2, 1, 8, 0), (1, 4, 1, 8, 0),
+               (2, 1, 1, 8, 0), (4, 2, 1, 4, 0)],
+    "synthetic": [(2, 1, 1, 0, 0), (1, 2, 1, 0, 0)],
+    "nash": [(1, 1, 1, 0, 0), (1, 4, 1, 0, 0)],
+}
+
+
+def rect_inputs(fn, m, n, dsize, dev):
+    if fn == "seqcmp":
+        x, y = workloads.seqcmp_inputs(m, n)
+        return (x, y), (_dev(x, dev), _dev(y, dev), None, None)
+    if fn == "synthetic":
+        u, v, top, left = workloads.synthetic_inputs(m, n, dsize)
+        return (u, v, top, left), (_dev(u, dev), _dev(v, dev), [_dev(top[d], dev) for d in range(dsize)],
+                                   [_dev(left[d], dev) for d in range(dsize)])
+    r, c, top, left = workloads.nash_inputs(m, n)
+    return (r, c, top, left), (_dev(r, dev), _dev(c, dev), [_dev(top[p], dev) for p in range(4)],
+                               [_dev(left[p], dev) for p in range(4)])
+
+
+def slab_parity_ok(cfg, k, w, d, impl, G, band_cols, strip=0, rows=64):
+    """G linked slabs of a small rectangular instance (rows x (G bands + a ragged tail)) against
+    the oracle (exact for integers, 1e-5 for floats)."""
+    cols = max(300, G * band_cols + 77)
+    host, _ = rect_inputs(cfg.fn, rows, cols, cfg.dsize, torch.device("cuda", 0))
+    want = oracle_grid(cfg.fn, host, cfg)
+    ngpu = torch.cuda.device_count()
+    ls = LocalSlabs(cfg.fn, rows, G, devices=[g % ngpu for g in range(G)], cols=cols, lane_cols=k, warps=w, skew=d,
+                    kernel=impl, strip=strip, **fn_kw(cfg))
+    try:
+        per = [rect_inputs(cfg.fn, rows, cols, cfg.dsize, torch.device("cuda", s.device))[1] for s in ls.slabs]
+        outs = ls.run(per)
+        ls.sync()
+        got = [np.concatenate([o[p].cpu().numpy() for o in outs], axis=1) for p in range(len(want))]
+    finally:
+        ls.close()
+    for g, o in zip(got, want):
+        o = np.asarray(o)
+        if o.dtype.kind == "f":
+            g = g.view(np.float32)
+            if not np.all(np.abs(g - o) <= 1e-5 * np.abs(o)):
+                return False
+        elif not np.array_equal(g.view(o.dtype), o):
+            return False
+    return True
+
+
 def sweep_slabs(cfg, reps, slabs):
-    """The gpu-count axis: the config's default tuning on G slabs (wall clock around the linked runs)."""
+    """The gpu-count axis: for every G, the config default plus SLAB_TUNINGS[fn] on G linked column
+    slabs, each point parity-gated on G slabs of a small instance, then timed (wall clock around the
+    linked runs).  With fewer physical GPUs than G the slabs are virtual (one GPU, each slab 1/G of
+    the resident CTAs): a point whose slabs together need more CTAs than the GPU holds at once is
+    marked 'ctas_exceed_sms' -- for one-CTA-per-SM kernels its time is not a prediction of G real
+    GPUs."""
     host, _ = inputs_for(cfg.fn, 16, cfg.dsize, torch.device("cuda", 0))
+    sms = torch.cuda.get_device_properties(0).multi_processor_count
     recs = []
     for G in slabs:
-        rec = {"slabs": G, "visible_gpus": torch.cuda.device_count(),
-               "placement": "virtual (one GPU)" if torch.cuda.device_count() < G else "one GPU per slab"}
-        try:
-            ms = time_slabs(cfg, 0, 0, 0, 0, host, G, reps)
-            rec.update(ms=round(ms, 4), gcups=round(cfg.dim * cfg.dim / ms / 1e6, 3))
-        except Exception as e:  # noqa: BLE001
-            rec["error"] = str(e)[:160]
-        recs.append(rec)
-        print(json.dumps(rec), flush=True)
+        for tun in [(0, 0, 0, 0, 0)] + SLAB_TUNINGS[cfg.fn]:
+            k, w, d, impl, st = tun
+            rec = {"slabs": G, "lane_cols": k, "warps": w, "skew": d, "kernel": impl, "strip": st,
+                   "visible_gpus": torch.cuda.device_count(),
+                   "placement": "virtual (one GPU)" if torch.cuda.device_count() < G else "one GPU per slab"}
+            try:
+                lay = [query(cfg.fn, cfg.dim, rank=g, ngpus=G, lane_cols=k, warps=w, skew=d, kernel=impl, strip=st,
+                             **fn_kw(cfg)) for g in range(G)]
+                rec.update(lane_cols=lay[0].lane_cols, warps=lay[0].warps, skew=lay[0].skew, strip=lay[0].strip,
+                           band_cols=lay[0].band_cols, bands_per_slab=[l_.nbands for l_ in lay])
+                if k and (lay[0].lane_cols, lay[0].warps, lay[0].skew) != (k, w, d):
+                    continue
+                rec["ctas_total"] = sum(l_.nbands for l_ in lay)
+                # virtual slabs share one GPU: with more bands than SMs, kernels that fit one CTA per
+                # SM (generation 8: ~199 KB of shared memory) make bands wait for a CTA, so the point
+                # does not predict G real GPUs (one-warp synthetic CTAs fit several per SM)
+                rec["sms"] = sms
+                rec["ctas_exceed_sms"] = rec["placement"].startswith("virtual") and rec["ctas_total"] > sms
+                if not slab_parity_ok(cfg, k, w, d, impl, G, lay[0].band_cols, st):
+                    rec["error"] = "parity"
+                else:
+                    ms = time_slabs(cfg, k, w, d, impl, host, G, reps, st)
+                    rec.update(ms=round(ms, 4), gcups=round(cfg.dim * cfg.dim / ms / 1e6, 3))
+            except Exception as e:  # noqa: BLE001
+                rec["error"] = str(e)[:160]
+            recs.append(rec)
+            print(json.dumps(rec), flush=True)
     return recs
 
 
@@ -182,18 +274,19 @@ def tune(cfg, reps, small, budget_s):
     sp = SEARCH[cfg.fn]
     points = []
     t_start = time.time()
-    for impl, k, w, d in itertools.product(sp["impl"], sp["k"], sp["w"], sp["d"]):
-        if not compiled(cfg, k, w, d, impl):
+    for impl, k, w, d, st in itertools.product(sp["impl"], sp["k"], sp["w"], sp["d"], sp["s"]):
+        if not compiled(cfg, k, w, d, impl, st):
             continue
+        rec = {"impl": impl, "k": k, "w": w, "d": d, "strip": st}
         if time.time() - t_start > budget_s:
-            points.append({"impl": impl, "k": k, "w": w, "d": d, "skipped": "time budget"})
+            rec["skipped"] = "time budget"
+            points.append(rec)
             continue
-        rec = {"impl": impl, "k": k, "w": w, "d": d}
         try:
-            if not parity_ok(cfg, k, w, d, impl, dev, small):
+            if not parity_ok(cfg, k, w, d, impl, dev, small, st):
                 rec["error"] = "parity mismatch vs oracle"
             else:
-                ms, nb = time_point(cfg, k, w, d, impl, devin, reps)
+                ms, nb = time_point(cfg, k, w, d, impl, devin, reps, st)
                 rec.update(ms=round(ms, 4), gcups=round(cfg.dim * cfg.dim / ms / 1e6, 3), nbands=nb)
         except Exception as e:  # noqa: BLE001 -- unsupported variants are part of the sweep
             rec["error"] = str(e)[:160]

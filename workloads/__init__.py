@@ -27,12 +27,17 @@ def unit_half_open_f32(rng: np.random.Generator, shape) -> np.ndarray:
     return ((k + (1 << 23)).astype(np.float64) * 2.0 ** -24).astype(np.float32)
 
 
+PROTEIN = b"ACDEFGHIKLMNPQRSTVWY"   # the 20 standard amino-acid one-letter codes
+
+
 def seqcmp_inputs(m: int, n: int | None = None, kind: str = "random", seed_x: int = SEED_X,
                   seed_y: int = SEED_Y, alphabet: int = 4, mutation: float = 0.10):
     """DNA-like residue codes in {0..alphabet-1} (uint8).
 
     kind: 'random' (x, y independent uniform), 'identical' (y = x), 'disjoint'
-    (x over {0,1}, y over {2,3}), 'mutated' (y = x with `mutation` of positions redrawn).
+    (x over {0,1}, y over {2,3}), 'mutated' (y = x with `mutation` of positions redrawn),
+    'protein' (ASCII amino-acid letters, PROTEIN), 'dna_ascii' (b"ACGT"), 'bytes' (any byte
+    value 0..255, including 0x80..0xff) -- the wf_params.alphabet = 0 inputs.
     """
     n = m if n is None else n
     rx, ry = _rng(seed_x), _rng(seed_y)
@@ -45,6 +50,13 @@ def seqcmp_inputs(m: int, n: int | None = None, kind: str = "random", seed_x: in
     elif kind == "disjoint":
         x = rx.integers(0, 2, size=m, dtype=np.uint8)
         y = (ry.integers(0, 2, size=n, dtype=np.uint8) + 2).astype(np.uint8)
+    elif kind in ("protein", "dna_ascii"):
+        letters = np.frombuffer(PROTEIN if kind == "protein" else b"ACGT", dtype=np.uint8)
+        x = letters[rx.integers(0, len(letters), size=m)]
+        y = letters[ry.integers(0, len(letters), size=n)]
+    elif kind == "bytes":
+        x = rx.integers(0, 256, size=m, dtype=np.uint8)
+        y = ry.integers(0, 256, size=n, dtype=np.uint8)
     elif kind == "mutated":
         base = rx.integers(0, alphabet, size=max(m, n), dtype=np.uint8)
         x = base[:m].copy()
