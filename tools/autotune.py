@@ -139,7 +139,7 @@ def compiled(cfg, k, w, d, impl, strip=0):
 def time_slabs(cfg, k, w, d, impl, host, G, reps, strip=0):
     """G column slabs of the same grid linked by the per-row P2P hand-off.  Virtual slabs (one
     GPU): device time between two events on the current stream, which gates every slab stream --
-    a ~2 ms device-side sleep ahead of the start event holds the slabs back until the host has
+    a ~10 ms device-side sleep ahead of the start event holds the slabs back until the host has
     enqueued all G launches, so host launch latency is not timed.  One GPU per slab: wall clock."""
     ngpu = torch.cuda.device_count()
     devices = [g % ngpu for g in range(G)]
@@ -159,7 +159,7 @@ def time_slabs(cfg, k, w, d, impl, host, G, reps, strip=0):
             if virtual:
                 cur = torch.cuda.current_stream()
                 e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-                torch.cuda._sleep(4_000_000)
+                torch.cuda._sleep(20_000_000)
                 e0.record(cur)
                 outs = ls.run(per, outs)   # every slab stream waits on cur (LocalSlabs.run)
                 for st in ls.streams:
