@@ -213,7 +213,11 @@ class LocalSlabs:
 
     devices: list of CUDA ordinals (len G).  Several slabs may share one device ("virtual
     GPUs"): they run concurrently on separate streams, each with 1/share of the
-    resident CTAs, and exchange edges through the same LL rings as real GPUs."""
+    resident CTAs, and exchange edges through the same rings as real GPUs.  Slabs are launched
+    in slab order, so when streams share a hardware queue a slab can only wait behind a LOWER
+    slab, which never waits on it -- no deadlock; but with 8 or more slabs per device set
+    CUDA_DEVICE_MAX_CONNECTIONS=32 before CUDA initialises, or a slab may start only after an
+    earlier slab's whole run (C4, 8 virtual slabs: 2.71 vs 2.01 ms)."""
 
     def __init__(self, fn, dim, ngpus: int, devices=None, **kw):
         devices = list(devices) if devices is not None else [torch.cuda.current_device()] * ngpus

@@ -2,6 +2,9 @@ import os
 import sys
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+# virtual-slab tests run up to 4 slab streams per device; keep every stream on its own hardware
+# queue (paper_conf_ppopp_mohantyc14_b200.wf.LocalSlabs)
+os.environ.setdefault("CUDA_DEVICE_MAX_CONNECTIONS", "32")
 if ROOT not in sys.path:
     sys.path.insert(0, ROOT)
 

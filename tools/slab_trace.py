@@ -14,6 +14,7 @@ import numpy as np
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
 os.environ["WF_TRACE"] = "1"
+os.environ.setdefault("CUDA_DEVICE_MAX_CONNECTIONS", "32")   # see LocalSlabs
 
 import torch  # noqa: E402
 

@@ -35,7 +35,7 @@ from paper_conf_ppopp_mohantyc14_b200.tuner import FNS, features  # noqa: E402
 def default_choice(fn, dim, tsize, dsize):
     """The library's fixed defaults (wf_api.cpp::defaults) as a (k, w, d, impl) tuple."""
     if fn == "seqcmp":
-        return (4, 2, 1, 4)
+        return (2, 4, 1, 8)   # generation 8, K = 2 x 4 warps
     if fn == "nash":
         return (1, 2, 1, 0)
     syn_pad_wins = dsize == 5 and tsize >= 1000
