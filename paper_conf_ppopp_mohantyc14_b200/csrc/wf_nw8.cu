@@ -60,8 +60,17 @@ namespace nw8 {
 #ifndef WF_NW8_U
 #define WF_NW8_U 16    // steps per lockstep block (A/B: 8 and 4 slower, profiles/r02_nw8_ab.txt)
 #endif
+#ifndef WF_NW8_HELPER_TMA
+// who issues the compute warps' TMA output stores: 0 = each compute warp's lane 0, 1 = the
+// helper warp, 2 = a separate storer warp (on another SM sub-partition than the helper)
+#define WF_NW8_HELPER_TMA 2
+#endif
+constexpr int kExtraWarps = WF_NW8_HELPER_TMA == 2 ? 2 : 1;   // warps besides the compute warps
 #ifndef WF_NW8_DPRE
-#define WF_NW8_DPRE 1  // blocks ahead the helper loads the inbound words (A/B 1 / 2 / 3: 1.96 / 2.02 / 2.06 ms)
+#define WF_NW8_DPRE 2  // blocks ahead the helper loads the inbound words (profiles/r02_nw8_ab.txt)
+#endif
+#ifndef WF_NW8_DIRECT_EAST
+#define WF_NW8_DIRECT_EAST 1   // the last compute warp stores its east words straight to the next band's ring
 #endif
 
 constexpr int RR = 128;        // slots per shared ring (power of 2, > 2U for every compiled U <= 32)
@@ -143,6 +152,14 @@ __device__ __forceinline__ int32_t lds32(uint32_t a) {
 }
 // predicated store: a divergent `if (lane == 31)` would wrap the following shuffles in a
 // reconvergence sequence
+__device__ __forceinline__ void stg128_if(bool p, int32_t* a, const int4& v) {
+  asm volatile("{ .reg .pred q; setp.ne.b32 q, %5, 0; @q st.volatile.global.v4.s32 [%0], {%1, %2, %3, %4}; }" ::"l"(a),
+               "r"(v.x), "r"(v.y), "r"(v.z), "r"(v.w), "r"(static_cast<int>(p)));
+}
+__device__ __forceinline__ void stg32_if(bool p, int32_t* a, int32_t v) {
+  asm volatile("{ .reg .pred q; setp.ne.b32 q, %2, 0; @q st.volatile.global.s32 [%0], %1; }" ::"l"(a), "r"(v),
+               "r"(static_cast<int>(p)));
+}
 __device__ __forceinline__ void sts32_if(bool p, uint32_t a, int32_t v) {
   asm volatile("{ .reg .pred q; setp.ne.b32 q, %2, 0; @q st.shared.s32 [%0], %1; }" ::"r"(a), "r"(v),
                "r"(static_cast<int>(p)));
@@ -178,7 +195,7 @@ struct Warp {
   using S = Smem<K, WARPS>;
   static constexpr int ROWB = S::ROWB;
   static constexpr int LAG = 32 + U;   // rows between consecutive warps (lockstep)
-  static constexpr int NT = (WARPS + 1) * 32;   // threads at the CTA barrier (compute warps + helper)
+  static constexpr int NT = (WARPS + kExtraWarps) * 32;   // threads at the CTA barrier (compute + helper warps)
   static_assert(U % 4 == 0 && 32 % U == 0, "block of U steps: multiple of 4, divides 32");
   static_assert(RR > 2 * U, "ring size");
   static_assert(SR * ROWB <= 65536, "staging slot arithmetic");
@@ -201,6 +218,9 @@ struct Warp {
   uint32_t lane_off;      // lane * 4K (byte offset of the lane's columns in a staged row)
   uint32_t ring_in;       // shared address of ring WI
   uint32_t ring_out;      // shared address of ring WI + 1
+  int32_t* gout;          // last warp (WF_NW8_DIRECT_EAST): the next band's / slab's global ring, row r at gout[r]
+  bool east_out;          // ... and there is one (not the last band of the last slab); lane 31 only
+  int32_t east_last;      // last warp: lane 31's east word of the current step
   uint32_t x_s;           // shared address of the x copy (x of row r at x_s + r - 1)
   int32_t best = 0, best_row = 0;   // LOCAL: best cell value of the lane and the first row reaching it
 
@@ -229,6 +249,15 @@ struct Warp {
     lane_off = uint32_t(lane) * 4 * K;
     ring_in = saddr(sm.ring) + uint32_t(WI) * RR * 4;
     ring_out = saddr(sm.ring) + uint32_t(WI + 1) * RR * 4;
+    gout = nullptr;
+    east_out = false;
+    if (WF_NW8_DIRECT_EAST && WI == WARPS - 1) {
+      int32_t* gbase = reinterpret_cast<int32_t*>(L.edge);
+      gout = (band + 1 < L.nbands) ? gbase + size_t(band + 1) * gring_stride(rows) + kGOff
+                                   : (L.next_edge ? reinterpret_cast<int32_t*>(L.next_edge) + kGOff : nullptr);
+      east_out = gout != nullptr;
+      east_out = east_out && is31;
+    }
     x_s = saddr(sm.x);
   }
 
@@ -269,7 +298,11 @@ struct Warp {
     }
     bool active = true;
     if constexpr (EDGE) active = row >= 1 && row <= rows;
-    sts32_if(is31 && active, rout, H[K - 1]);   // east hand-off: lane 31's row s - 31
+    if (WF_NW8_DIRECT_EAST && WI == WARPS - 1) {
+      east_last = H[K - 1];   // block() stores 4 rows at a time into the next band's ring
+    } else {
+      sts32_if(is31 && active, rout, H[K - 1]);   // east hand-off: lane 31's row s - 31
+    }
     if constexpr (LOCAL) {   // best cell: strict > keeps the first row reaching the value
       int32_t rm = H[0];
 #pragma unroll
@@ -319,12 +352,20 @@ struct Warp {
     }
     const uint32_t s_off = uint32_t(s0 - lane) * ROWB;    // staging offset of the lane's row at step s0+1
     const uint32_t xnext = x_s + uint32_t(s0 + U - lane);  // x of the lane's rows in the next block
+    int32_t eq[4];
 #pragma unroll
     for (int u = 0; u < U; ++u) {
       // lane 31's rows s0-30+u: quads of ring slots aligned at s0-30+4q (s0 - 28 = 0 mod 4)
       const uint32_t rout = ring_out + slot(s0 - 30 + (u & ~3)) + 4u * (u & 3);
       step<EDGE>(s0 + 1 + u, xc[u], in[u], s_off + uint32_t(u * ROWB), rout);
       asm volatile("ld.shared.u8 %0, [%1];" : "=r"(xc[u]) : "r"(xnext + uint32_t(u)));
+      if constexpr (WF_NW8_DIRECT_EAST && WI == WARPS - 1) {
+        // the band's east column, 4 rows per 16-byte store (rows s0-30+u-3 .. s0-30+u, an aligned
+        // quad of the next band's / slab's global ring; rows <= 0 or > rows land in its slack,
+        // which is never read)
+        eq[u & 3] = east_last;
+        if ((u & 3) == 3) stg128_if(east_out, gout + (s0 - 33 + u), make_int4(eq[0], eq[1], eq[2], eq[3]));
+      }
     }
   }
 
@@ -340,10 +381,17 @@ struct Warp {
     __syncwarp();
   }
 
-  // end of the block s0+1 .. s0+U: TMA store of a completed 32-row box, then the CTA barrier
+  // end of the block s0+1 .. s0+U, then the CTA barrier.  When rows e-63 .. e-32 are complete
+  // (lane 31 passed them) their 32-row box is stored: with WF_NW8_HELPER_TMA the warp only
+  // fences its staged rows into the async proxy and the helper issues the TMA store after the
+  // barrier (Helper::store_boxes); otherwise lane 0 issues it here.
   __device__ __forceinline__ void after_block(int s0) {
     const int e = s0 + U;   // last local step done
-    if (e % 32 == 0 && e >= 64) publish(e - 63);   // rows e-63 .. e-32 complete (lane 31 passed them)
+#if WF_NW8_HELPER_TMA
+    if (e % 32 == 0 && e >= 64) fence_proxy_async_smem();   // the helper / storer warp stores the box
+#else
+    if (e % 32 == 0 && e >= 64) publish(e - 63);
+#endif
     wf_jitter(1 + WI);
     cta_bar<NT>();
   }
@@ -428,13 +476,16 @@ template <int K, int WARPS, bool LOCAL, int U>
 struct Helper {
   using S = Smem<K, WARPS>;
   static constexpr int LAG = 32 + U;
-  static constexpr int NT = (WARPS + 1) * 32;
+  static constexpr int NT = (WARPS + kExtraWarps) * 32;
 
   const SweepLaunch& L;
+  const CUtensorMap* tmap;
   const int band, lane;
   int rows;
   bool inbound, outbound, mine;
   uint32_t ring0, ringW;
+  uint32_t stage0;        // shared address of compute warp 0's staging ring
+  int elast;              // every compute warp's last local block end (ceil(Tw / U) U)
   int32_t* gin;
   int32_t* gout;
   int4 emptyq;
@@ -443,9 +494,12 @@ struct Helper {
   bool failed = false;
   Watchdog wd;
 
-  __device__ __forceinline__ Helper(const SweepLaunch& L_, const S& sm, int band_, int lane_, bool first)
-      : L(L_), band(band_), lane(lane_) {
+  __device__ __forceinline__ Helper(const SweepLaunch& L_, const CUtensorMap* tm, const S& sm, int band_, int lane_,
+                                    bool first)
+      : L(L_), tmap(tm), band(band_), lane(lane_) {
     rows = L.rows;
+    stage0 = saddr(sm.stage);
+    elast = ((rows + 31 + U - 1) / U) * U;
     mine = lane < U / 4;
     ring0 = saddr(sm.ring);
     ringW = saddr(sm.ring) + uint32_t(WARPS) * RR * 4;
@@ -495,6 +549,39 @@ struct Helper {
     }
   }
 
+  // TMA stores of the 32-row boxes the compute warps completed at CTA step B (warp w's local
+  // step e = B - w LAG, e = 0 mod 32, 64 <= e <= its last block end), one commit group per
+  // call; the box of e is read out of its staging slots before the barrier at CTA step
+  // B + 64, after which warp w may rewrite them (hence wait_group.read 3 with one group per
+  // block).  Lane 0 only: bulk async-groups are per thread.
+  __device__ __forceinline__ void store_boxes(int B) {
+    if (lane != 0) return;
+#pragma unroll
+    for (int w = 0; w < WARPS; ++w) {
+      const int e = B - w * LAG;
+      if (e >= 64 && (e & 31) == 0 && e <= elast) {
+        const int r0 = e - 63;
+        tma_store_2d(tmap, stage0 + uint32_t(w) * SR * S::ROWB + uint32_t((r0 - 1) & (SR - 1)) * S::ROWB,
+                     band * L.band_w + w * 32 * K, r0 - 1);
+      }
+    }
+    bulk_commit();
+    bulk_wait_read<3>();
+  }
+
+  // the storer warp (WF_NW8_HELPER_TMA == 2): the CTA's barrier sequence with only the stores
+  __device__ __forceinline__ void run_storer() {
+    const int Tc = rows + 31 + (WARPS - 1) * LAG;
+    cta_bar<NT>();
+    int B = 0;
+    for (; B < Tc; B += U) {
+      store_boxes(B);
+      cta_bar<NT>();
+    }
+    store_boxes(B);
+    if (lane == 0) bulk_wait_all();
+  }
+
   __device__ __forceinline__ void run() {
     const int Tw = rows + 31;
     const int Tc = Tw + (WARPS - 1) * LAG;
@@ -537,20 +624,28 @@ struct Helper {
       deliver(0);
     }
     cta_bar<NT>();   // warp 0's first block reads what the prologue stored
-    for (int B = 0; B < Tc; B += U) {
+    int B = 0;
+    for (; B < Tc; B += U) {
       // B = CTA step of this block's start; warp 0's current block has local start s0 = B
       wf_jitter(9);
       if (inbound && B + U < Tw) deliver(B + U);   // warp 0's next block starts at local step B + U
-      if (outbound && B >= U) {       // the last warp's block that ended at this block's start
+      if (!WF_NW8_DIRECT_EAST && outbound && B >= U) {   // the last warp's block that ended at this block's start
         const int s0 = B - U - Ll;
         if (s0 >= 0 && s0 < Tw) forward(s0);
       }
+#if WF_NW8_HELPER_TMA == 1
+      store_boxes(B);
+#endif
       cta_bar<NT>();
     }
-    if (outbound) {
+    if (!WF_NW8_DIRECT_EAST && outbound) {
       const int s0 = ((Tc + U - 1) / U) * U - U - Ll;   // the last warp's final block
       if (s0 >= 0 && s0 < Tw) forward(s0);
     }
+#if WF_NW8_HELPER_TMA == 1
+    store_boxes(B);   // boxes completed by the final block (the compute warps store the rest)
+    if (lane == 0) bulk_wait_all();
+#endif
     if (inbound && band == 0 && !L.first_slab && L.ack_prev) {   // predecessor slab may reuse this ring
       __threadfence_system();
       if (lane == 0) st_relaxed_sys_u32(L.ack_prev, L.epoch);
@@ -576,13 +671,14 @@ __device__ __forceinline__ void dispatch(const SweepLaunch& L, const CUtensorMap
       dispatch<K, WARPS, WI + 1, LOCAL, U>(L, tm, sm, band, warp, lane, first);
     }
   } else {
-    Helper<K, WARPS, LOCAL, U> h(L, sm, band, lane, first);
-    h.run();
+    Helper<K, WARPS, LOCAL, U> h(L, tm, sm, band, lane, first);
+    if (WF_NW8_HELPER_TMA == 2 && warp == WARPS + 1) h.run_storer();
+    else h.run();
   }
 }
 
 template <int K, int WARPS, bool LOCAL, int U>
-__global__ void __launch_bounds__((WARPS + 1) * 32, 1)
+__global__ void __launch_bounds__((WARPS + kExtraWarps) * 32, 1)
     nw8_kernel(const __grid_constant__ SweepLaunch L, const __grid_constant__ CUtensorMap tmap) {
   using S = Smem<K, WARPS>;
   extern __shared__ __align__(16) unsigned char nw8_smem_raw[];
@@ -620,7 +716,7 @@ cudaError_t launch(const SweepLaunch& L, cudaStream_t s, size_t smem) {
   auto kfn = L.local ? nw8_kernel<K, WARPS, true, U> : nw8_kernel<K, WARPS, false, U>;
   e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
-  kfn<<<L.grid, (WARPS + 1) * 32, smem, s>>>(L, tmap);
+  kfn<<<L.grid, (WARPS + kExtraWarps) * 32, smem, s>>>(L, tmap);
   return cudaGetLastError();
 }
 
@@ -628,7 +724,7 @@ cudaError_t launch(const SweepLaunch& L, cudaStream_t s, size_t smem) {
 // hand-off and per helper message
 template <int K, int WARPS, bool LOCAL, int U = kU>
 Variant make() {
-  return Variant{WF_FN_SEQCMP, LOCAL ? 1 : 0, K, WARPS, 1, (WARPS + 1) * 32, Smem<K, WARPS>::bytes,
+  return Variant{WF_FN_SEQCMP, LOCAL ? 1 : 0, K, WARPS, 1, (WARPS + kExtraWarps) * 32, Smem<K, WARPS>::bytes,
                  reinterpret_cast<const void*>(nw8_kernel<K, WARPS, LOCAL, U>), &launch<K, WARPS, U>, 8, {}, U};
 }
 
