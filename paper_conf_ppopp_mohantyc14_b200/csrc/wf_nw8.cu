@@ -66,8 +66,8 @@ namespace nw8 {
 #define WF_NW8_HELPER_TMA 2
 #endif
 constexpr int kExtraWarps = WF_NW8_HELPER_TMA == 2 ? 2 : 1;   // warps besides the compute warps
-#ifndef WF_NW8_DPRE
-#define WF_NW8_DPRE 2  // blocks ahead the helper loads the inbound words (profiles/r02_nw8_ab.txt)
+#ifndef WF_NW8_DPRE_ROWS
+#define WF_NW8_DPRE_ROWS 32  // rows ahead the helper loads the inbound words (profiles/r02_nw8_ab.txt)
 #endif
 #ifndef WF_NW8_DIRECT_EAST
 #define WF_NW8_DIRECT_EAST 1   // the last compute warp stores its east words straight to the next band's ring
@@ -489,7 +489,7 @@ struct Helper {
   int32_t* gin;
   int32_t* gout;
   int4 emptyq;
-  static constexpr int DP = WF_NW8_DPRE;
+  static constexpr int DP = WF_NW8_DPRE_ROWS / U > 0 ? WF_NW8_DPRE_ROWS / U : 1;   // blocks of lead
   int4 pre[DP];       // inbound quads of the next DP blocks (pre[0] = the next to deliver)
   bool failed = false;
   Watchdog wd;
@@ -575,6 +575,7 @@ struct Helper {
     cta_bar<NT>();
     int B = 0;
     for (; B < Tc; B += U) {
+      wf_jitter(10);
       store_boxes(B);
       cta_bar<NT>();
     }

@@ -25,15 +25,17 @@ REGIONS = {
         ("wf_nw.cuh", 786, 834, "kernel entry / exit"),
     ],
     "nw8": [
-        ("wf_nw8.cu", 242, 292, "compute: cell step (DPX chain, staging STS, east ring STS)"),
-        ("wf_nw8.cu", 293, 331, "compute: block (x codes, west ring LDS)"),
-        ("wf_nw8.cu", 332, 343, "compute: TMA store publish"),
-        ("wf_nw8.cu", 344, 350, "compute: block barrier (lockstep wait)"),
-        ("wf_nw8.cu", 351, 394, "compute: lag / drain barriers, run loop"),
-        ("wf_nw8.cu", 176, 241, "compute: setup"),
-        ("wf_nw8.cu", 398, 415, "helper: spin on a stale global quad (stall on flag)"),
-        ("wf_nw8.cu", 427, 559, "helper warp: global ring in/out + its barriers"),
-        ("wf_nw8.cu", 561, 611, "kernel entry / dispatch / exit"),
+        ("wf_nw8.cu", 271, 325, "compute: cell step (DPX chain, staging STS, east hand-off)"),
+        ("wf_nw8.cu", 326, 372, "compute: block (x codes, west ring LDS, east quads)"),
+        ("wf_nw8.cu", 373, 387, "compute: TMA store publish (tail only)"),
+        ("wf_nw8.cu", 388, 398, "compute: block barrier (lockstep wait)"),
+        ("wf_nw8.cu", 399, 442, "compute: lag / drain barriers, run loop"),
+        ("wf_nw8.cu", 193, 270, "compute: setup"),
+        ("wf_nw8.cu", 446, 463, "helper: spin on a stale global quad (stall on flag)"),
+        ("wf_nw8.cu", 557, 585, "storer warp: TMA output stores + its barriers"),
+        ("wf_nw8.cu", 476, 556, "helper warp: inbound ring + its barriers"),
+        ("wf_nw8.cu", 586, 655, "helper warp: inbound ring + its barriers"),
+        ("wf_nw8.cu", 657, 708, "kernel entry / dispatch / exit"),
     ],
     "syn": [
         ("wf_syn.cu", 236, 248, "compute: dependency wait (wait_ctr: west hand-off / ring slot)"),

@@ -6,7 +6,7 @@
     per step and slow-path counts (wf_nw8.cu trace slots).
 
     python tools/nw8_probe.py parity 777:2:2 777:2:4 ...
-    WF_TRACE=1 python tools/nw8_probe.py trace [dim] [lane_cols] [warps]
+    WF_TRACE=1 python tools/nw8_probe.py trace [dim] [lane_cols] [warps] [strip]
     WF_PROBE_LIB=tools/abl_out/libwf_X.so ...      (an A/B build of tools/xbuild8.sh)
 """
 from __future__ import annotations
@@ -49,7 +49,7 @@ def parity(specs):
                   g[r0, max(0, c0 - 3):c0 + 3])
 
 
-def trace(dim=32768, k=0, w=0):
+def trace(dim=32768, k=0, w=0, strip=0):
     import torch
     import workloads
     from paper_conf_ppopp_mohantyc14_b200.wf import Wavefront
@@ -62,6 +62,8 @@ def trace(dim=32768, k=0, w=0):
         kw["lane_cols"] = k
     if w:
         kw["warps"] = w
+    if strip:
+        kw["strip"] = strip
     with Wavefront("seqcmp", dim, **kw) as wf:
         out = wf.alloc_out()
         for _ in range(3):
