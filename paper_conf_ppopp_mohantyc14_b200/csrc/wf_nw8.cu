@@ -223,6 +223,7 @@ struct Warp {
   int32_t east_last;      // last warp: lane 31's east word of the current step
   uint32_t x_s;           // shared address of the x copy (x of row r at x_s + r - 1)
   int32_t best = 0, best_row = 0;   // LOCAL: best cell value of the lane and the first row reaching it
+  int32_t vrow;           // NW: r c of the lane's first virtual row r = -lane (0 for SW)
 
   __device__ __forceinline__ Warp(const SweepLaunch& L_, const CUtensorMap* tm, const S& sm, int band_, int lane_)
       : L(L_), tmap(tm), band(band_), lane(lane_), is31(lane_ == 31) {
@@ -236,14 +237,25 @@ struct Warp {
     const uint8_t* y = static_cast<const uint8_t*>(L.col_in);
     wcol = band * L.band_w + WI * 32 * K;
     const int jb = L.c0 + wcol + lane * K;   // global 0-based first column of the lane
+    // NW: lane l starts at step 1 on row 1 - l.  Instead of predicating every state update of the
+    // ramp-up steps (rows <= 0), the row-0 boundary is extended to virtual rows r <= 0 by
+    // V(r, j) = j g + r c with c = max(1, g, max(match, mismatch) - g): V is a fixed point of the
+    // recurrence (N + g <= V since g <= c; NW + s <= V since s - g <= c; W + g = V), so a lane
+    // that starts from row -l's V values and receives V as its west input reproduces V on its
+    // virtual rows and reaches row 0 = the true boundary, for any scores (
+    // checked over the ABI scoring range by tests/test_nw_virtual_rows.py).
+    // SW keeps the predicated ramp (its floor 0 has no such extension).
+    const int32_t vc_ = max(1, max(gap, max(mmatch, mmis) - gap));
+    vrow = LOCAL ? 0 : -lane * vc_;                                          // V(-lane, j) - j g
 #pragma unroll
     for (int m = 0; m < K; ++m) {
       const bool vc = jb + m < L.c1;
       ycode[m] = vc ? static_cast<uint32_t>(__ldg(y + jb + m)) : 0x100u;   // never equal to a code
-      N[m] = (vc && !LOCAL) ? (jb + m + 1) * gap : 0;                      // H[0][j] = j g (NW), 0 (SW)
+      N[m] = LOCAL ? 0 : (jb + m + 1) * gap + vrow;                         // H[0][j] = j g (NW; V(-lane, j)), 0 (SW)
     }
-    NWc = (!LOCAL) ? jb * gap : 0;                                          // H[0][jb]
-    src = 0;
+    NWc = (!LOCAL) ? jb * gap + vrow : 0;                                   // H[0][jb] (NW: V(-lane, jb))
+    // what this lane hands its east neighbour at step 1: its east value of row -lane (NW: V)
+    src = LOCAL ? 0 : (jb + K) * gap + vrow;
     srcl = (lane + 31) & 31;
     stage_s = saddr(sm.stage) + uint32_t(WI) * SR * ROWB;
     lane_off = uint32_t(lane) * 4 * K;
@@ -409,25 +421,35 @@ struct Warp {
     int B = 0;
     for (; B < Lw; B += U) cta_bar<NT>();   // before this warp's first block (its lag)
     // row 1's word (stored before this barrier) and the x codes of the first block
-    src = is31 ? (BOUND ? (LOCAL ? 0 : gap) : lds32(ring_in + slot(1))) : 0;
+    if (is31) src = BOUND ? (LOCAL ? 0 : gap) : lds32(ring_in + slot(1));
     const long long c1 = clock64();
     if (tr) tr[1] = globaltimer();
     uint32_t xc[U];
     load_x(0, xc);
     int s0 = 0;   // local steps s0+1 .. s0+U of the block starting at CTA step B = s0 + Lw
-    // ramp-up (lane 31 not yet on row 1) and steady blocks, then the drain
-    for (; s0 < 31 && s0 < Tw; s0 += U) {
-      block<true>(s0, xc);
-      after_block(s0);
-    }
+    if constexpr (!LOCAL) {
+      // NW: the ramp-up runs through the virtual rows (constructor) and the drain's rows > rows
+      // are clipped by the tensor bounds and never read, so every block is a steady block
 #pragma unroll 1
-    for (; s0 + U <= rows; s0 += U) {
-      block<false>(s0, xc);
-      after_block(s0);
-    }
-    for (; s0 < Tw; s0 += U) {
-      block<true>(s0, xc);
-      after_block(s0);
+      for (; s0 < Tw; s0 += U) {
+        block<false>(s0, xc);
+        after_block(s0);
+      }
+    } else {
+      // SW: ramp-up (lane 31 not yet on row 1) and steady blocks, then the drain
+      for (; s0 < 31 && s0 < Tw; s0 += U) {
+        block<true>(s0, xc);
+        after_block(s0);
+      }
+#pragma unroll 1
+      for (; s0 + U <= rows; s0 += U) {
+        block<false>(s0, xc);
+        after_block(s0);
+      }
+      for (; s0 < Tw; s0 += U) {
+        block<true>(s0, xc);
+        after_block(s0);
+      }
     }
     for (B = s0 + Lw; B < Tc; B += U) cta_bar<NT>();   // the other warps' drain
     // the rows not yet stored: from the last published box on (s0 = ceil(Tw / U) * U)
@@ -492,6 +514,7 @@ struct Helper {
   static constexpr int DP = WF_NW8_DPRE_ROWS / U > 0 ? WF_NW8_DPRE_ROWS / U : 1;   // blocks of lead
   int4 pre[DP];       // inbound quads of the next DP blocks (pre[0] = the next to deliver)
   bool failed = false;
+  unsigned nslow = 0;     // WF_TRACE: blocks whose inbound quads were not all there when delivered
   Watchdog wd;
 
   __device__ __forceinline__ Helper(const SweepLaunch& L_, const CUtensorMap* tm, const S& sm, int band_, int lane_,
@@ -530,6 +553,7 @@ struct Helper {
     int4 v = pre[0];
     const bool st = need && quad_stale(v, r, rows);
     if (!failed && __any_sync(FULL, st)) {
+      ++nslow;
       const Slow4 w = slow_quad(L, gin + r, r, rows, need);
       failed = w.failed != 0;
       if (need) v = w.v;
@@ -647,6 +671,7 @@ struct Helper {
     store_boxes(B);   // boxes completed by the final block (the compute warps store the rest)
     if (lane == 0) bulk_wait_all();
 #endif
+    if (L.trace && lane == 0) L.trace[size_t(band) * kTraceSlots + 8 * WARPS + 4] = nslow;   // helper slot
     if (inbound && band == 0 && !L.first_slab && L.ack_prev) {   // predecessor slab may reuse this ring
       __threadfence_system();
       if (lane == 0) st_relaxed_sys_u32(L.ack_prev, L.epoch);

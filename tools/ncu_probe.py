@@ -13,6 +13,8 @@ reps = int(sys.argv[4]) if len(sys.argv) > 4 else 3
 tsize = int(sys.argv[5]) if len(sys.argv) > 5 else 0
 dsize = int(sys.argv[6]) if len(sys.argv) > 6 else 0
 cols = int(sys.argv[7]) if len(sys.argv) > 7 else 0
+kernel = int(sys.argv[8]) if len(sys.argv) > 8 else 0
+strip = int(sys.argv[9]) if len(sys.argv) > 9 else 0
 dev = torch.device("cuda", 0)
 t = lambda a: torch.from_numpy(np.ascontiguousarray(a)).to(dev)
 if fn == "seqcmp":
@@ -25,7 +27,7 @@ else:
     u, v, top, left = workloads.synthetic_inputs(dim, cols or dim, dsize)
     ins = (t(u), t(v), [t(top[i]) for i in range(dsize)], [t(left[i]) for i in range(dsize)])
     kw = dict(tsize=tsize, dsize=dsize)
-wf = Wavefront(fn, dim, cols=cols, lane_cols=k, warps=w, skew=d, watchdog_cycles=1 << 42, **({"alphabet": 4} if fn == "seqcmp" else {}), **kw)
+wf = Wavefront(fn, dim, cols=cols, lane_cols=k, warps=w, skew=d, watchdog_cycles=1 << 42, kernel=kernel, strip=strip, **({"alphabet": 4} if fn == "seqcmp" else {}), **kw)
 out = wf.alloc_out()
 for _ in range(reps):
     wf.run(*ins, out=out)

@@ -6,7 +6,7 @@
     per step and slow-path counts (wf_nw8.cu trace slots).
 
     python tools/nw8_probe.py parity 777:2:2 777:2:4 ...
-    WF_TRACE=1 python tools/nw8_probe.py trace [dim] [lane_cols] [warps] [strip]
+    WF_TRACE=1 python tools/nw8_probe.py trace [dim] [lane_cols] [warps] [strip] [kernel]
     WF_PROBE_LIB=tools/abl_out/libwf_X.so ...      (an A/B build of tools/xbuild8.sh)
 """
 from __future__ import annotations
@@ -25,18 +25,19 @@ if os.environ.get("WF_PROBE_LIB"):   # A/B builds from tools/xbuild8.sh (the pro
     _abi.LIB_PATH = os.path.abspath(os.environ["WF_PROBE_LIB"])
 
 
-def parity(specs):
+def parity(specs, kernel=0):
     import oracle
     import workloads
     from _gpu_helpers import run_gpu
     for spec in specs:
-        dim, k, w = (int(v) for v in spec.split(":"))
+        dim, k, w = (int(v) for v in spec.split(":")[:3])
+        kern = int(spec.split(":")[3]) if spec.count(":") >= 3 else kernel
         x, y = workloads.seqcmp_inputs(dim, dim, seed_x=dim, seed_y=dim + 1)
         H = oracle.seqcmp(x, y, 1, -1, -1)
-        (g,) = run_gpu("seqcmp", dim, (x, y), lane_cols=k, warps=w, skew=1)
+        (g,) = run_gpu("seqcmp", dim, (x, y), lane_cols=k, warps=w, skew=1, kernel=kern)
         bad = np.argwhere(H != g)
         bw = 32 * k * w
-        print(f"dim={dim} K={k} W={w}: {len(bad)} mismatches", flush=True)
+        print(f"dim={dim} K={k} W={w} kernel={kern}: {len(bad)} mismatches", flush=True)
         if len(bad):
             cols = np.unique(bad[:, 1])
             rows = np.unique(bad[:, 0])
@@ -49,7 +50,7 @@ def parity(specs):
                   g[r0, max(0, c0 - 3):c0 + 3])
 
 
-def trace(dim=32768, k=0, w=0, strip=0):
+def trace(dim=32768, k=0, w=0, strip=0, kernel=0):
     import torch
     import workloads
     from paper_conf_ppopp_mohantyc14_b200.wf import Wavefront
@@ -64,6 +65,8 @@ def trace(dim=32768, k=0, w=0, strip=0):
         kw["warps"] = w
     if strip:
         kw["strip"] = strip
+    if kernel:
+        kw["kernel"] = kernel
     with Wavefront("seqcmp", dim, **kw) as wf:
         out = wf.alloc_out()
         for _ in range(3):
@@ -76,7 +79,7 @@ def trace(dim=32768, k=0, w=0, strip=0):
     W = lay.warps
     t0 = int(tr[:, 0].min())
     print(f"dim={dim} K={lay.lane_cols} W={W} bands={lay.nbands} run {ms:.3f} ms")
-    steps = dim + 31
+    steps = (dim + 1) // 2 + 31 if kernel == 9 else dim + 31
     rows_out = []
     for b in range(lay.nbands):
         for w_ in range(W):
@@ -96,7 +99,9 @@ def trace(dim=32768, k=0, w=0, strip=0):
           f" CTA hops {np.mean([d[i] for i in range(len(d)) if (i + 1) % W == 0]) / 1e3:.3f} us")
     cyc = np.array([r[5] for r in rows_out])
     print(f"sweep cycles per step: median {np.median(cyc):.1f}, min {cyc.min():.1f}, max {cyc.max():.1f}")
-    print("slow bodies total", int(sum(r[6] for r in rows_out)))
+    hs = tr[:, 8 * W + 4].astype(np.int64)
+    print("helper slow-path blocks per band: bands 1,2,64,last:", [int(hs[b]) for b in (1, 2, lay.nbands // 2, lay.nbands - 1)],
+          "mean", float(hs[1:].mean()) if lay.nbands > 1 else 0.0, "of", (dim + 31) // 16, "blocks")
 
 
 if __name__ == "__main__":
