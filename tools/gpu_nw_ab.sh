@@ -1,5 +1,9 @@
-WF_TRACE=1 WF_PROBE_LIB=tools/abl_out/libwf_old.so timeout 300 python tools/nw8_probe.py trace 32768 > gpurun_out/ab1_trace_old.txt 2>&1
-WF_TRACE=1 timeout 300 python tools/nw8_probe.py trace 32768 > gpurun_out/ab1_trace_new.txt 2>&1
-WF_TRACE=1 WF_PROBE_LIB=tools/abl_out/libwf_dpre48.so timeout 300 python tools/nw8_probe.py trace 32768 > gpurun_out/ab1_trace_d48.txt 2>&1
-WF_TRACE=1 WF_PROBE_LIB=tools/abl_out/libwf_dpre64.so timeout 300 python tools/nw8_probe.py trace 32768 > gpurun_out/ab1_trace_d64.txt 2>&1
-timeout 900 python tools/ab_time.py --rounds 4 old=tools/abl_out/libwf_old.so new=- d48=tools/abl_out/libwf_dpre48.so d64=tools/abl_out/libwf_dpre64.so > gpurun_out/ab1.txt 2>&1
+# same-box A/B of NW builds: parity subset of the in-tree build, WF_TRACE timelines and interleaved timing
+# usage: bash tools/gpu_nw_ab.sh NAME=lib ...   (lib '-' = in-tree)
+timeout 1200 python -m pytest tests/test_parity_gpu.py tests/test_multiproc_gpu.py tests/test_abi_gpu.py -m gpu -x -q -k "seqcmp or smith or abi or multiproc or link or connect" > gpurun_out/ab_tests.txt 2>&1; echo "tests rc=$?" >> gpurun_out/ab_tests.txt
+for nb in "$@"; do
+  n=${nb%%=*}; l=${nb#*=}
+  if [ "$l" = "-" ]; then WF_TRACE=1 timeout 300 python tools/nw8_probe.py trace 32768 > gpurun_out/ab_trace_$n.txt 2>&1
+  else WF_TRACE=1 WF_PROBE_LIB=$l timeout 300 python tools/nw8_probe.py trace 32768 > gpurun_out/ab_trace_$n.txt 2>&1; fi
+done
+timeout 900 python tools/ab_time.py --rounds 4 "$@" > gpurun_out/ab.txt 2>&1
