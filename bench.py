@@ -304,11 +304,14 @@ def run_ours(args, cfg):
         v = getattr(args, k)
         if v:
             tun[k] = v
-    w = Wavefront(cfg.fn, cfg.dim, rank=rank, device=local, ngpus=world, **fn_kwargs(cfg), **tun)
+    staged = world > 1 and args.transport == "nccl"
+    w = Wavefront(cfg.fn, cfg.dim, rank=rank, device=local, ngpus=world, transport=args.transport, **fn_kwargs(cfg), **tun)
     lay = w.layout
-    if world > 1:
+    if world > 1 and not staged:
         from paper_conf_ppopp_mohantyc14_b200.dist import connect_slab
         connect_slab(w, rank, world)   # all-gather of edge-ring IPC handles, wf_connect to g-1 / g+1
+    if staged:   # host-staged slab edges over NCCL send/recv (include/wf.h wf_edge_*)
+        from paper_conf_ppopp_mohantyc14_b200.dist import staged_run
 
     inputs = host_inputs(cfg)
     if cfg.fn == "seqcmp":
@@ -323,6 +326,11 @@ def run_ours(args, cfg):
     row_in, col_in = [p.to(dev) for p in pinned]
     out = w.alloc_out()
     stream = torch.cuda.current_stream()
+
+    def sweep(r_in, c_in):
+        if staged:
+            return staged_run(w, (r_in, c_in, tops, lefts), rank, world, stream=stream, out=out)
+        return w.run(r_in, c_in, tops, lefts, out=out, stream=stream)
     slab_cells = cfg.dim * lay.width
     total_cells = cfg.dim * cfg.dim
     footprint = lay.bytes_out
@@ -335,7 +343,7 @@ def run_ours(args, cfg):
         torch.cuda.synchronize()
 
     for _ in range(args.warmup):
-        w.run(row_in, col_in, tops, lefts, out=out, stream=stream)
+        sweep(row_in, col_in)
     barrier()
     w.sync()
 
@@ -348,14 +356,15 @@ def run_ours(args, cfg):
             if flush:
                 flush_buf.fill_(i)
             ev[i][0].record(stream)
-            w.run(row_in, col_in, tops, lefts, out=out, stream=stream)
+            sweep(row_in, col_in)
             ev[i][1].record(stream)
         t_end.record(stream)
         torch.cuda.synchronize()
         barrier()
     w.sync()
     launch_ms = [a.elapsed_time(b) for a, b in ev]
-    step_ms_local = (sum(launch_ms) if flush else t_start.elapsed_time(t_end)) / args.steps
+    # staged slabs run one after another: a rank's window includes its wait for the predecessor
+    step_ms_local = (sum(launch_ms) if flush and not staged else t_start.elapsed_time(t_end)) / args.steps
     avg_launch_ms = sum(launch_ms) / len(launch_ms)
     if world > 1:
         from paper_conf_ppopp_mohantyc14_b200.dist import max_over_ranks
@@ -374,7 +383,7 @@ def run_ours(args, cfg):
     for _ in range(e2e_steps):
         r_d = pinned[0].to(dev, non_blocking=True)
         c_d = pinned[1].to(dev, non_blocking=True)
-        o = w.run(r_d, c_d, tops, lefts, out=out, stream=stream)
+        o = sweep(r_d, c_d)
         for f in range(lay.nplanes):
             res_host[f].copy_(o[f][-1].view(torch.int32), non_blocking=True)
     e1.record(stream)
@@ -398,7 +407,7 @@ def run_ours(args, cfg):
         for _ in range(reps):
             r_d = pinned[0].to(dev, non_blocking=True)
             c_d = pinned[1].to(dev, non_blocking=True)
-            o = w.run(r_d, c_d, tops, lefts, out=out, stream=stream)
+            o = sweep(r_d, c_d)
             for f in range(lay.nplanes):
                 host_grid[f].copy_(o[f], non_blocking=True)
         g1.record(stream)
@@ -425,6 +434,7 @@ def run_ours(args, cfg):
                        "dsize": cfg.dsize, "lane_cols": lay.lane_cols, "warps": lay.warps, "skew": lay.skew,
                        "band_cols": lay.band_cols, "nbands_per_slab": lay.nbands,
                        "parallelism": f"column slabs x{world}" if world > 1 else "1 GPU",
+                       "transport": args.transport if world > 1 else None,
                        "l2": ("explicit 252 MiB L2 flush between steps (footprint < 2x L2)" if flush else
                               f"outputs {footprint / 2**30:.2f} GiB per GPU > 126 MB L2; no flush needed")},
             "gpu_launches": args.steps * world,
@@ -459,6 +469,9 @@ def main():
     ap.add_argument("--lane-cols", dest="lane_cols", type=int, default=0)
     ap.add_argument("--warps", type=int, default=0)
     ap.add_argument("--skew", type=int, default=0)
+    ap.add_argument("--transport", choices=["p2p", "nccl"], default="p2p",
+                    help="N > 1: slab-edge transport (p2p = the sweep's own NVLink stores, pipelined; "
+                         "nccl = host-staged send/recv fallback, slabs in sequence)")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--e2e-grid", dest="e2e_grid", action="store_true", default=True)
     ap.add_argument("--no-e2e-grid", dest="e2e_grid", action="store_false")

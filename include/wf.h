@@ -93,8 +93,13 @@ typedef struct {
   int32_t ngpus;        /* slabs (column blocks), 1..8; see wf_dist */
   int32_t match, mismatch, gap;  /* SEQCMP scores, each in [-64, 64]; defaults used if all three 0 */
   int32_t local;        /* SEQCMP: 0 = global (Needleman-Wunsch), 1 = local (Smith-Waterman) */
-  uint32_t transport;   /* wf_transport for ngpus > 1: only WF_TRANSPORT_P2P is built; NCCL ->
-                           WF_EUNSUPPORTED */
+  uint32_t transport;   /* wf_transport for ngpus > 1:
+                           P2P (default) = the sweep stores the slab's east edge straight into the
+                           successor's ring (wf_link_local / wf_connect), pipelined row block by row block;
+                           NCCL = the host-staged fallback for systems without peer access: each slab
+                           writes its east edge into a library buffer, the caller moves it with the
+                           process group's send/recv (wf_edge_export / wf_edge_import) and slab g+1 runs
+                           after slab g -- the paper's host-staged halo swap, not pipelined */
   uint32_t max_ctas;    /* 0 = all resident CTAs; else an upper bound (tests of the band loop) */
   uint64_t watchdog_cycles; /* spin budget per dependency wait (SM clock cycles); 0 = default: the larger of
                                2^32 and 4x the expected pipeline fill (bands x slabs x 64 rows x the
@@ -208,6 +213,23 @@ wf_status wf_ipc_handle(struct wf_ctx* c, void* handle);
  * stored into its ring over NVLink.  WF_EINVAL if a required handle is missing, WF_ECOMM if
  * a handle cannot be opened. */
 wf_status wf_connect(struct wf_ctx* c, const void* prev_handle, const void* next_handle);
+
+/* transport = WF_TRANSPORT_NCCL ("data elements have to be first transferred to the
+ * host ... then to respective destination GPUs"; SURVEY.md §8(a) a8 "Fallback: NCCL send/recv"):
+ * the slab-edge message of a staged context.
+ *   wf_edge_bytes:  size of one message (the byte image of a band-0 edge ring; identical on all
+ *                   ranks of one problem and tuning).
+ *   wf_edge_export: rank < world-1: enqueue on `cuda_stream` a copy of the east edge written by
+ *                   this slab's last wf_run into `dst` (device or pinned host memory, bytes from
+ *                   wf_edge_bytes, caller-owned); call after wf_run on the same stream.
+ *   wf_edge_import: rank > 0: enqueue a copy of the predecessor's exported message `src` into this
+ *                   slab's inbound ring; call before wf_run on the same stream.
+ * Every rank issues the same sequence of wf_run calls.  WF_ESTATE for a context that is not
+ * staged (transport P2P, or a single slab) or for the wrong end of the chain; WF_EINVAL for
+ * NULL pointers; WF_ECUDA if the copy cannot be enqueued. */
+wf_status wf_edge_bytes(const struct wf_ctx* c, size_t* bytes);
+wf_status wf_edge_export(struct wf_ctx* c, void* dst, void* cuda_stream);
+wf_status wf_edge_import(struct wf_ctx* c, const void* src, void* cuda_stream);
 
 /* SEQCMP local = 1 (Smith-Waterman): the best local
  * alignment score of this slab's columns and its cell, the first in row-major order holding

@@ -23,7 +23,7 @@ WF_TRANSPORT_P2P, WF_TRANSPORT_NCCL = 0, 1
 # every symbol include/wf.h declares (checked by tests/test_abi.py)
 EXPORTS = ("wf_query", "wf_create", "wf_run", "wf_sync", "wf_destroy", "wf_last_error", "wf_link_local",
            "wf_ipc_handle", "wf_connect", "wf_last_run_ms", "wf_abi_version", "wf_build_info", "wf_debug_trace",
-           "wf_local_best")
+           "wf_local_best", "wf_edge_bytes", "wf_edge_export", "wf_edge_import")
 
 
 class WfParams(ctypes.Structure):
@@ -93,8 +93,12 @@ def lib() -> ctypes.CDLL:
         L.wf_abi_version.restype = ctypes.c_int32
         L.wf_build_info.argtypes = []
         L.wf_build_info.restype = ctypes.c_char_p
+        L.wf_edge_bytes.argtypes = [P, ctypes.POINTER(ctypes.c_size_t)]
+        L.wf_edge_export.argtypes = [P, P, P]
+        L.wf_edge_import.argtypes = [P, P, P]
         for name in ("wf_query", "wf_create", "wf_run", "wf_sync", "wf_destroy", "wf_link_local",
-                     "wf_ipc_handle", "wf_connect", "wf_last_run_ms", "wf_local_best"):
+                     "wf_ipc_handle", "wf_connect", "wf_last_run_ms", "wf_local_best", "wf_edge_bytes",
+                     "wf_edge_export", "wf_edge_import"):
             getattr(L, name).restype = ctypes.c_int
         _lib = L
     return _lib

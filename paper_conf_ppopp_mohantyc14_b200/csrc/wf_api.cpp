@@ -49,6 +49,9 @@ struct wf_ctx {
   cudaEvent_t ev0 = nullptr, ev1 = nullptr;
   cudaEvent_t ev2 = nullptr;               // after the error-word copy of the last run
   bool ran = false;
+  bool staged = false;                     // transport NCCL, world > 1: host-staged slab edges
+  void* stage = nullptr;                   // rank < world-1: this slab's outbound edge ring (staged)
+  size_t stage_bytes = 0;                  // one slab-edge message (a band-0 ring image)
   std::string msg;
 };
 
@@ -133,10 +136,6 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   const int G = p->ngpus ? p->ngpus : 1;
   if (rank < 0 || rank >= G) return fail(c, WF_EINVAL, "rank=%d out of range for ngpus=%d", rank, G);
   if (p->transport > WF_TRANSPORT_NCCL) return fail(c, WF_EINVAL, "transport=%u unknown", p->transport);
-  // The slab hand-off is P2P stores issued by the sweep itself; a host-driven
-  // NCCL exchange is not built, and is refused rather than silently ignored.
-  if (p->transport == WF_TRANSPORT_NCCL)
-    return fail(c, WF_EUNSUPPORTED, "transport=NCCL is not built (P2P hand-off only, DESIGN.md §8)");
   // strip = rows per hand-off block (the band-to-band and slab-to-slab message); selectable
   // for generation 8 among its compiled blocks, fixed (0) for the other generations
   if (p->strip < 0 || p->strip > 65535) return fail(c, WF_EINVAL, "strip=%d out of range 0..65535", p->strip);
@@ -347,6 +346,15 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
     c->ack = static_cast<unsigned*>(c->base);
     c->edge = reinterpret_cast<unsigned long long*>(static_cast<char*>(c->base) + kCtrlBytes);
   }
+  // transport NCCL: the last band stores its east edge into a local outbound ring (same layout as
+  // a band-0 inbound ring) which the caller ships with send/recv (wf_edge_export / import)
+  c->staged = p->transport == WF_TRANSPORT_NCCL && c->world > 1;
+  c->stage_bytes = (wfk::edge_stride(p->dim) + 64) * pl.nf * sizeof(unsigned long long);
+  if (e == cudaSuccess && c->staged && c->rank < c->world - 1) {
+    e = cudaMalloc(&c->stage, c->stage_bytes);
+    if (e == cudaSuccess) e = cudaMemset(c->stage, 0x80, c->stage_bytes);
+    if (e == cudaSuccess) c->next_edge = static_cast<unsigned long long*>(c->stage);
+  }
   if (e == cudaSuccess) e = cudaMalloc(&c->err, sizeof(int));
   if (e == cudaSuccess) e = cudaMemset(c->err, 0, sizeof(int));
   if (e == cudaSuccess) e = cudaMallocHost(&c->err_host, sizeof(int));
@@ -394,6 +402,7 @@ wf_status wf_destroy(wf_ctx* c) {
   if (c->next_ipc_base) cudaIpcCloseMemHandle(c->next_ipc_base);
   if (c->prev_ipc_base) cudaIpcCloseMemHandle(c->prev_ipc_base);
   if (c->base) cudaFree(c->base);
+  if (c->stage) cudaFree(c->stage);
   if (c->err) cudaFree(c->err);
   if (c->err_host) cudaFreeHost(c->err_host);
   if (c->lane_best) cudaFree(c->lane_best);
@@ -410,6 +419,8 @@ wf_status wf_destroy(wf_ctx* c) {
 
 wf_status wf_link_local(wf_ctx* prev, wf_ctx* next) {
   if (!prev || !next) return fail(prev, WF_EINVAL, "wf_link_local: NULL context");
+  if (prev->staged || next->staged)
+    return fail(prev, WF_ESTATE, "wf_link_local: transport NCCL slabs exchange edges with wf_edge_export / wf_edge_import");
   if (next->rank != prev->rank + 1 || next->world != prev->world)
     return fail(prev, WF_EINVAL, "wf_link_local: ranks %d -> %d are not consecutive slabs", prev->rank, next->rank);
   if (prev->nf != next->nf || prev->p.dim != next->p.dim || prev->p.fn != next->p.fn ||
@@ -484,6 +495,7 @@ static wf_status open_ipc(wf_ctx* c, const void* handle, void** out) {
 
 wf_status wf_connect(wf_ctx* c, const void* prev_handle, const void* next_handle) {
   if (!c) return fail(c, WF_EINVAL, "wf_connect: NULL context");
+  if (c->staged) return fail(c, WF_ESTATE, "wf_connect: transport NCCL slabs exchange edges with wf_edge_export / wf_edge_import");
   // the slabs' per-run acks and rings are epoch-paired: every rank connects before its first run
   // (all ranks then issue the same sequence of wf_run calls)
   if (c->ran || c->epoch != 0)
@@ -569,8 +581,10 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   L.pitch = io->out_pitch;
   L.edge = c->edge;
   L.next_edge = c->next_edge;
-  L.ack_self = c->ack;
-  L.ack_prev = c->ack_prev;
+  // staged slabs: the host orders each run's edge message after the producer and before the
+  // consumer on the streams, so there is no cross-run ack between slabs
+  L.ack_self = c->staged ? nullptr : c->ack;
+  L.ack_prev = c->staged ? nullptr : c->ack_prev;
   L.first_slab = c->rank == 0;
   // a device error of the previous run that has already completed (its error word was copied to
   // pinned host memory behind it) is reported here, once, without blocking (include/wf.h)
@@ -627,6 +641,37 @@ wf_status wf_sync(wf_ctx* c) {
                 (unsigned long long)c->watchdog, c->epoch);
   }
   return WF_OK;
+}
+
+wf_status wf_edge_bytes(const wf_ctx* c, size_t* bytes) {
+  if (!c || !bytes) return fail(nullptr, WF_EINVAL, "wf_edge_bytes: NULL argument");
+  if (!c->staged) return fail(const_cast<wf_ctx*>(c), WF_ESTATE, "wf_edge_bytes: not a transport NCCL slab");
+  *bytes = c->stage_bytes;
+  return WF_OK;
+}
+
+static wf_status edge_copy(wf_ctx* c, void* dst, const void* src, void* stream, const char* what) {
+  int prev = -1;
+  cudaGetDevice(&prev);
+  if (prev != c->device) cudaSetDevice(c->device);
+  cudaError_t e = cudaMemcpyAsync(dst, src, c->stage_bytes, cudaMemcpyDefault, static_cast<cudaStream_t>(stream));
+  if (prev >= 0 && prev != c->device) cudaSetDevice(prev);
+  if (e != cudaSuccess) return cuda_fail(c, e, what);
+  return WF_OK;
+}
+
+wf_status wf_edge_export(wf_ctx* c, void* dst, void* cuda_stream) {
+  if (!c || !dst) return fail(c, WF_EINVAL, "wf_edge_export: NULL argument");
+  if (!c->staged || c->rank >= c->world - 1)
+    return fail(c, WF_ESTATE, "wf_edge_export: only a transport NCCL slab with a successor exports its edge");
+  return edge_copy(c, dst, c->stage, cuda_stream, "wf_edge_export");
+}
+
+wf_status wf_edge_import(wf_ctx* c, const void* src, void* cuda_stream) {
+  if (!c || !src) return fail(c, WF_EINVAL, "wf_edge_import: NULL argument");
+  if (!c->staged || c->rank == 0)
+    return fail(c, WF_ESTATE, "wf_edge_import: only a transport NCCL slab with a predecessor imports an edge");
+  return edge_copy(c, c->edge, src, cuda_stream, "wf_edge_import");
 }
 
 wf_status wf_debug_trace(wf_ctx* c, void* host, size_t bytes, int32_t* slots_per_band) {

@@ -80,3 +80,48 @@ def connect_slab(w, rank: int, world: int, group=None) -> None:
     that all ranks agree on problem, tuning and slab adjacency (ValueError otherwise)."""
     prev, nxt = exchange_handles(w.ipc_handle(), slab_fingerprint(w), rank, world, group)
     w.connect(prev, nxt)
+
+
+def staged_sequence(rank: int, world: int, nbytes: int, *, recv, edge_import, run, edge_export, send):
+    """The host-staged slab chain of one run (transport="nccl"): rank g > 0 receives rank g-1's
+    edge message (nbytes) and imports it before its sweep; rank g < G-1 exports its east edge
+    after the sweep and sends it to g+1.  The callables carry the data movement, so the ordering
+    is testable with gloo on CPU (tests/test_multirank_gloo.py).  Returns run()'s result."""
+    if rank > 0:
+        edge_import(recv(nbytes))
+    out = run()
+    if rank < world - 1:
+        send(edge_export(nbytes))
+    return out
+
+
+def staged_run(w, args, rank: int, world: int, group=None, comm_device=None, stream=None, out=None):
+    """One wf_run of a transport="nccl" slab (SURVEY.md §8(a) a8 fallback): receive
+    rank-1's edge message, import it, sweep, export this slab's east edge and send it to rank+1.
+    The slabs therefore run one after another -- the host-staged halo swap of P:247-253 over the
+    process group (NCCL on the GPU box; gloo with CPU buffers in the tests), not pipelined.
+
+    comm_device: where the message lives for send/recv (None = the slab's CUDA device, as NCCL
+    needs; "cpu" for gloo).  Returns the output planes."""
+    dev = torch.device("cuda", w.device)
+    cdev = dev if comm_device is None else torch.device(comm_device)
+
+    def recv(n):
+        msg = torch.empty(n, dtype=torch.uint8, device=cdev)
+        dist.recv(msg, src=rank - 1, group=group)
+        return msg
+
+    def edge_import(msg):
+        w.edge_import(msg if msg.device == dev else msg.to(dev), stream)
+
+    def edge_export(n):
+        buf = torch.empty(n, dtype=torch.uint8, device=dev)
+        w.edge_export(buf, stream)
+        (torch.cuda.current_stream(dev) if stream is None else stream).synchronize()   # the send reads buf
+        return buf
+
+    def send(buf):
+        dist.send(buf if cdev == dev else buf.to(cdev), dst=rank + 1, group=group)
+
+    return staged_sequence(rank, world, w.edge_bytes(), recv=recv, edge_import=edge_import,
+                           run=lambda: w.run(*args, out=out, stream=stream), edge_export=edge_export, send=send)

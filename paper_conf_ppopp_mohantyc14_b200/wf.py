@@ -182,6 +182,28 @@ class Wavefront:
         with torch.cuda.device(self.device):
             check(_abi.lib().wf_connect(self._ctx, bufs[0], bufs[1]), self._ctx)
 
+    # ---- transport = "nccl": host-staged slab edges (wf_edge_export / wf_edge_import)
+    def edge_bytes(self) -> int:
+        n = ctypes.c_size_t()
+        check(_abi.lib().wf_edge_bytes(self._ctx, ctypes.byref(n)), self._ctx)
+        return int(n.value)
+
+    def edge_export(self, dst: torch.Tensor, stream=None) -> None:
+        """Enqueue a copy of the east edge of this slab's last run into `dst` (>= edge_bytes())."""
+        if dst.numel() * dst.element_size() < self.edge_bytes() or not dst.is_contiguous():
+            raise ValueError("edge_export: dst must be contiguous and hold edge_bytes() bytes")
+        with torch.cuda.device(self.device):
+            check(_abi.lib().wf_edge_export(self._ctx, ctypes.c_void_p(dst.data_ptr()),
+                                            ctypes.c_void_p(_stream_handle(stream))), self._ctx)
+
+    def edge_import(self, src: torch.Tensor, stream=None) -> None:
+        """Enqueue a copy of the predecessor's exported edge `src` into this slab's inbound ring."""
+        if src.numel() * src.element_size() < self.edge_bytes() or not src.is_contiguous():
+            raise ValueError("edge_import: src must be contiguous and hold edge_bytes() bytes")
+        with torch.cuda.device(self.device):
+            check(_abi.lib().wf_edge_import(self._ctx, ctypes.c_void_p(src.data_ptr()),
+                                            ctypes.c_void_p(_stream_handle(stream))), self._ctx)
+
     def close(self) -> None:
         if getattr(self, "_ctx", None) is not None and self._ctx.value:
             _abi.lib().wf_destroy(self._ctx)

@@ -68,11 +68,18 @@ def test_query_rejects_bad_params_naming_the_field(kw, field):
     assert field in str(e)
 
 
-def test_unbuilt_nccl_transport_is_refused():
-    # the slab hand-off is the sweep's own P2P store; an NCCL transport is not
-    # built and must not be accepted and silently ignored
-    e = _err("seqcmp", 256, ngpus=2, transport="nccl")
-    assert e.status == _abi.WF_EUNSUPPORTED and "transport" in str(e)
+def test_nccl_transport_is_accepted_and_edge_calls_validate():
+    """transport = NCCL is the host-staged fallback (include/wf.h wf_edge_*):
+    the planner accepts it, and the edge calls reject NULL arguments without a GPU."""
+    lay = query("seqcmp", 1024, ngpus=2, transport="nccl")
+    assert lay.col_begin == 0 and lay.col_end > 0
+    L = _abi.lib()
+    n = ctypes.c_size_t()
+    assert L.wf_edge_bytes(None, ctypes.byref(n)) == _abi.WF_EINVAL
+    assert L.wf_edge_export(None, None, None) == _abi.WF_EINVAL
+    assert L.wf_edge_import(None, None, None) == _abi.WF_EINVAL
+    e = _err("seqcmp", 1024, ngpus=2, transport=7)
+    assert e.status == _abi.WF_EINVAL and "transport" in str(e)
 
 
 def test_strip_axis():

@@ -38,18 +38,26 @@ def _worker(rank, world, port, fn, dim, kw, reps, q):
         from paper_conf_ppopp_mohantyc14_b200 import dist as wdist
         from paper_conf_ppopp_mohantyc14_b200.wf import Wavefront
         dev = torch.device("cuda", 0)
+        staged = kw.get("transport") == "nccl"
         w = Wavefront(fn, dim, rank=rank, device=0, ngpus=world, watchdog_cycles=1 << 40, **kw)
-        wdist.connect_slab(w, rank, world)
+        if not staged:
+            wdist.connect_slab(w, rank, world)
         t = lambda a: torch.from_numpy(np.ascontiguousarray(a)).to(dev)  # noqa: E731
         if fn == "seqcmp":
             x, y = workloads.seqcmp_inputs(dim, dim)
             args = (t(x), t(y), None, None)   # col_in / top cover the whole grid (include/wf.h)
+        elif fn == "nash":
+            r_, c_, top, left = workloads.nash_inputs(dim)
+            args = (t(r_), t(c_), [t(top[p]) for p in range(4)], [t(left[p]) for p in range(4)])
         else:
             u, v, top, left = workloads.synthetic_inputs(dim, dim, kw["dsize"])
             args = (t(u), t(v), [t(top[d]) for d in range(kw["dsize"])], [t(left[d]) for d in range(kw["dsize"])])
         outs = []
-        for _ in range(reps):   # re-runs exercise the cross-run ack of the edge ring
-            out = w.run(*args)
+        for _ in range(reps):   # re-runs exercise the cross-run ack / the ring reset of the edge
+            if staged:   # host-staged edges over the process group (gloo: CPU message buffers)
+                out = wdist.staged_run(w, args, rank, world, comm_device="cpu")
+            else:
+                out = w.run(*args)
             w.sync()
             outs.append([o.cpu().numpy().copy() for o in out])
         gathered = [None] * world
@@ -104,3 +112,54 @@ def test_two_process_ipc_slabs_synthetic():
                 assert np.all(np.abs(g - want[p]) <= 1e-5 * np.abs(want[p]))
             else:
                 assert np.array_equal(g, want[p])
+
+
+# ---- transport = "nccl": the host-staged fallback (include/wf.h wf_edge_*; SURVEY.md §8(a) a8,
+# §4.2-4c: "the NCCL fallback checked against the P2P path: grids must be identical")
+def _gathered_grid(gathered, rep, plane, world=2):
+    return np.concatenate([gathered[r][rep][plane] for r in range(world)], axis=1)
+
+
+@pytest.mark.parametrize("kw", [dict(alphabet=4), dict(alphabet=4, kernel=4), dict(local=1)],
+                         ids=["nw_gen8", "nw_gen4", "sw"])
+def test_staged_transport_seqcmp_equals_p2p_and_oracle(kw):
+    import oracle
+    import workloads
+    dim = 1100
+    staged = _run("seqcmp", dim, dict(kw, transport="nccl"), reps=2)
+    p2p = _run("seqcmp", dim, dict(kw), reps=1)
+    x, y = workloads.seqcmp_inputs(dim, dim)
+    H = oracle.seqcmp(x, y, 1, -1, -1, local=kw.get("local", 0))
+    for rep in range(2):
+        g = _gathered_grid(staged, rep, 0)
+        assert np.array_equal(g, _gathered_grid(p2p, 0, 0))
+        assert np.array_equal(g, H)
+
+
+def test_staged_transport_synthetic_equals_p2p():
+    import oracle
+    import workloads
+    dim = 600
+    kw = dict(tsize=10, dsize=2)
+    staged = _run("synthetic", dim, dict(kw, transport="nccl"), reps=2)
+    p2p = _run("synthetic", dim, kw, reps=1)
+    u, v, top, left = workloads.synthetic_inputs(dim, dim, 2)
+    i0, i1, f = oracle.synthetic(u, v, top, left, 10)
+    want = [i0, i1, f[0], f[1]]
+    for rep in range(2):
+        for p in range(4):
+            g = _gathered_grid(staged, rep, p)
+            assert np.array_equal(g.view(np.uint32), _gathered_grid(p2p, 0, p).view(np.uint32))
+            assert np.array_equal(g.view(np.uint32), want[p].view(np.uint32))
+
+
+def test_staged_transport_nash_equals_oracle():
+    import oracle
+    import workloads
+    dim = 200
+    staged = _run("nash", dim, dict(tsize=16, dsize=4, transport="nccl"), reps=2)
+    r, c, top, left = workloads.nash_inputs(dim)
+    ref = oracle.nash(r, c, top, left, nstrat=16)
+    for rep in range(2):
+        for p in range(4):
+            assert np.array_equal(_gathered_grid(staged, rep, p), ref[p])

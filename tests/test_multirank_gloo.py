@@ -99,3 +99,66 @@ def test_check_fingerprints_single_process():
                      ([(prob, tun, (5, 40)), (prob, tun, (40, 100))], "starts at column")):
         with pytest.raises(ValueError, match=msg):
             check_fingerprints(fps)
+
+
+def _staged_worker(rank, world, port, q):
+    """transport="nccl" host sequencing (dist.staged_sequence) over gloo: each rank's 'sweep' adds
+    its rank to every byte of the message it imported, so the last rank sees the chain's sum only
+    if every message was received, imported, run, exported and sent in order."""
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        from paper_conf_ppopp_mohantyc14_b200 import dist as wdist
+        state = {"in": torch.zeros(64, dtype=torch.uint8), "ring": None, "log": []}
+
+        def recv(n):
+            m = torch.empty(n, dtype=torch.uint8)
+            dist.recv(m, src=rank - 1)
+            state["log"].append("recv")
+            return m
+
+        def edge_import(m):
+            state["in"] = m.clone()
+            state["log"].append("import")
+
+        def run():   # a pure function of this run's inputs, like the sweep
+            state["ring"] = state["in"] + (rank + 1)
+            state["log"].append("run")
+            return state["ring"].clone()
+
+        def edge_export(n):
+            state["log"].append("export")
+            return state["ring"][:n].clone()
+
+        def send(m):
+            dist.send(m, dst=rank + 1)
+            state["log"].append("send")
+
+        outs = [wdist.staged_sequence(rank, world, 64, recv=recv, edge_import=edge_import, run=run,
+                                      edge_export=edge_export, send=send) for _ in range(2)]
+        q.put((rank, (state["log"], [int(o[0]) for o in outs])))
+    except Exception as e:  # noqa: BLE001
+        q.put((rank, repr(e)))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("world", [2, 3])
+def test_staged_transport_sequence_gloo(world):
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_staged_worker, args=(r, world, port, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    res = dict(q.get(timeout=300) for _ in range(world))
+    for p in procs:
+        p.join(timeout=60)
+    for r in range(world):
+        assert not isinstance(res[r], str), res[r]
+        log, vals = res[r]
+        one = (["recv", "import"] if r > 0 else []) + ["run"] + (["export", "send"] if r < world - 1 else [])
+        assert log == one * 2
+        # run k of rank r sees the sum 1 + 2 + ... + (r + 1) (each run re-imports a fresh message)
+        assert vals == [sum(range(1, r + 2))] * 2
