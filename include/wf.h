@@ -114,7 +114,15 @@ typedef struct {
                            at skew 1), 8 = plane-split wf_syn (dsize 2..8, lane_cols = warps = skew = 1:
                            one warp per float item on the same 32 columns).  Other combinations
                            -> WF_EUNSUPPORTED */
-  int32_t reserved[4];  /* must be zero */
+  int32_t halo;         /* NEXT-4 comparison variant (PAPER.md P:238-255, P:289-296,
+                           Table 3): columns each slab g > 0 recomputes redundantly west of its own
+                           (an overlap of whole bands: a multiple of the band width); slab g then takes
+                           its west input from slab g-1's column c0 - halo - 1 instead of c0 - 1, and the
+                           overlap's cells go to a library scratch plane (outputs are unchanged).  SEQCMP
+                           global alignment with the generation-8 sweep, ngpus > 1 only; 0 = none.
+                           WF_EINVAL if not a positive multiple of the band width or if a slab has no
+                           band to spare; WF_EUNSUPPORTED for other functions / generations */
+  int32_t reserved[3];  /* must be zero */
 } wf_params;
 
 /* Distribution: which slab this context computes.

@@ -33,7 +33,8 @@ class WfParams(ctypes.Structure):
                 ("ngpus", ctypes.c_int32), ("match", ctypes.c_int32), ("mismatch", ctypes.c_int32),
                 ("gap", ctypes.c_int32), ("local", ctypes.c_int32), ("transport", ctypes.c_uint32),
                 ("max_ctas", ctypes.c_uint32), ("watchdog_cycles", ctypes.c_uint64),
-                ("alphabet", ctypes.c_int32), ("kernel", ctypes.c_int32), ("reserved", ctypes.c_int32 * 4)]
+                ("alphabet", ctypes.c_int32), ("kernel", ctypes.c_int32), ("halo", ctypes.c_int32),
+                ("reserved", ctypes.c_int32 * 3)]
 
 
 class WfDist(ctypes.Structure):

@@ -25,6 +25,9 @@ struct wf_ctx {
   int rank = 0, world = 1, device = 0, share = 1;
   int nf = 1, nbound = 0;
   int c0 = 0, c1 = 0;
+  int cc0 = 0, halo_bands = 0, export_band = 0;   // NEXT-4 halo (Plan)
+  void* halo_out = nullptr;                // overlap bands' scratch plane (rows x halo_pitch int32)
+  int64_t halo_pitch = 0;
   int k = 4, warps = 2, skew = 2, band_w = 256, nbands = 1;
   int grid = 1;
   int smem = 0;
@@ -78,6 +81,7 @@ wf_status cuda_fail(wf_ctx* c, cudaError_t e, const char* what) {
 
 struct Plan {
   int nf, nbound, k, warps, skew, band_w, c0, c1, nbands;
+  int cc0, halo_bands, export_band;   // NEXT-4 halo: first computed column, overlap bands, exporting band
   int impl;   // kernel generation actually used (wf_params.kernel, or the default's)
   int strip;  // wf_params.strip (0 = the generation's default block)
   int match, mismatch, gap;
@@ -128,8 +132,9 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
     return fail(c, WF_EINVAL, "kernel=%d must be 0 (default), 4, 7 or 8", p->kernel);
   if (p->fn == WF_FN_SEQCMP && p->kernel == 7)
     return fail(c, WF_EUNSUPPORTED, "kernel=7: SEQCMP has generations 4 and 8 (the per-row v7 kernel was retired, DESIGN.md §12)");
-  for (int i = 0; i < 4; ++i)
+  for (int i = 0; i < 3; ++i)
     if (p->reserved[i]) return fail(c, WF_EINVAL, "reserved[%d] must be 0", i);
+  if (p->halo < 0) return fail(c, WF_EINVAL, "halo=%d must be >= 0", p->halo);
   if (p->alphabet < 0 || p->alphabet > 8) return fail(c, WF_EINVAL, "alphabet=%d out of range 0..8", p->alphabet);
   if (p->alphabet != 0 && p->fn != WF_FN_SEQCMP) return fail(c, WF_EINVAL, "alphabet applies to SEQCMP only");
   if (p->ngpus < 0 || p->ngpus > 8) return fail(c, WF_EINVAL, "ngpus=%d out of range 1..8", p->ngpus);
@@ -200,6 +205,28 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   pl.c1 = (int)(b1 * pl.band_w < cols ? b1 * pl.band_w : cols);
   if (pl.c1 <= pl.c0) return fail(c, WF_EINVAL, "ngpus=%d leaves slab %d empty (cols=%d, band=%d)", G, rank, cols, pl.band_w);
   pl.nbands = (pl.c1 - pl.c0 + pl.band_w - 1) / pl.band_w;
+  pl.cc0 = pl.c0;
+  pl.halo_bands = 0;
+  pl.export_band = pl.nbands - 1;
+  if (p->halo) {
+    // NEXT-4: slab g > 0 recomputes m = halo / band_w whole bands west of its own; slab g < G-1
+    // exports the east edge of its band nbands-1-m (the column slab g+1's overlap starts after)
+    if (p->fn != WF_FN_SEQCMP || p->local || !(pl.impl == 0 || pl.impl == 8) || pl.skew != 1 ||
+        wfk::variant_strip(p->fn, 0, pl.k, pl.warps, pl.skew, pl.impl, pl.strip) == 0)
+      return fail(c, WF_EUNSUPPORTED, "halo: global SEQCMP with the generation-8 sweep only");
+    if (G < 2) return fail(c, WF_EINVAL, "halo=%d needs ngpus > 1", p->halo);
+    if (p->halo % pl.band_w) return fail(c, WF_EINVAL, "halo=%d must be a multiple of the band width %d", p->halo, pl.band_w);
+    const int m = p->halo / pl.band_w;
+    const int own = pl.nbands;
+    if (own <= m)
+      return fail(c, WF_EINVAL, "halo=%d: every slab needs more than %d bands (slab %d has %d)", p->halo, m, rank, own);
+    if (rank > 0) {
+      pl.cc0 = pl.c0 - p->halo;
+      pl.halo_bands = m;
+      pl.nbands = own + m;
+    }
+    pl.export_band = pl.nbands - 1 - m;
+  }
   *out = pl;
   return WF_OK;
 }
@@ -276,6 +303,9 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   c->nf = pl.nf;
   c->nbound = pl.nbound;
   c->c0 = pl.c0;
+  c->cc0 = pl.cc0;
+  c->halo_bands = pl.halo_bands;
+  c->export_band = pl.export_band;
   c->c1 = pl.c1;
   c->k = pl.k;
   c->warps = pl.warps;
@@ -355,6 +385,10 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
     if (e == cudaSuccess) e = cudaMemset(c->stage, 0x80, c->stage_bytes);
     if (e == cudaSuccess) c->next_edge = static_cast<unsigned long long*>(c->stage);
   }
+  if (e == cudaSuccess && c->halo_bands > 0) {   // NEXT-4: the overlap bands' cells (discarded)
+    c->halo_pitch = (int64_t)c->halo_bands * c->band_w;
+    e = cudaMalloc(&c->halo_out, (size_t)c->halo_pitch * p->dim * sizeof(int32_t));
+  }
   if (e == cudaSuccess) e = cudaMalloc(&c->err, sizeof(int));
   if (e == cudaSuccess) e = cudaMemset(c->err, 0, sizeof(int));
   if (e == cudaSuccess) e = cudaMallocHost(&c->err_host, sizeof(int));
@@ -403,6 +437,7 @@ wf_status wf_destroy(wf_ctx* c) {
   if (c->prev_ipc_base) cudaIpcCloseMemHandle(c->prev_ipc_base);
   if (c->base) cudaFree(c->base);
   if (c->stage) cudaFree(c->stage);
+  if (c->halo_out) cudaFree(c->halo_out);
   if (c->err) cudaFree(c->err);
   if (c->err_host) cudaFreeHost(c->err_host);
   if (c->lane_best) cudaFree(c->lane_best);
@@ -426,7 +461,8 @@ wf_status wf_link_local(wf_ctx* prev, wf_ctx* next) {
   if (prev->nf != next->nf || prev->p.dim != next->p.dim || prev->p.fn != next->p.fn ||
       prev->p.cols != next->p.cols || prev->p.tsize != next->p.tsize || prev->p.dsize != next->p.dsize ||
       prev->p.local != next->p.local || prev->impl != next->impl || prev->k != next->k ||
-      prev->warps != next->warps || prev->skew != next->skew || prev->strip != next->strip)
+      prev->warps != next->warps || prev->skew != next->skew || prev->strip != next->strip ||
+      prev->p.halo != next->p.halo)
     return fail(prev, WF_EINVAL, "wf_link_local: contexts describe different problems or tunings");
   if (prev->c1 != next->c0)
     return fail(prev, WF_EINVAL, "wf_link_local: slab %d ends at column %d but slab %d starts at %d", prev->rank,
@@ -561,6 +597,11 @@ wf_status wf_run(wf_ctx* c, const wf_io* io, void* cuda_stream) {
   L.best_out = c->best_out;
   L.c0 = c->c0;
   L.c1 = c->c1;
+  L.cc0 = c->cc0;
+  L.halo_bands = c->halo_bands;
+  L.export_band = c->export_band;
+  L.halo_out = c->halo_out;
+  L.halo_pitch = c->halo_pitch;
   L.match = p.match;
   L.mismatch = p.mismatch;
   L.gap = p.gap;

@@ -12,7 +12,12 @@ namespace wfk {
 struct SweepLaunch {
   // problem
   int32_t fn, rows, cols, tsize, dsize;
-  int32_t c0, c1;                 // slab interior columns [c0, c1), 0-based
+  int32_t c0, c1;                 // slab interior columns [c0, c1), 0-based (the output planes' columns)
+  int32_t cc0;                    // first computed column: c0 - halo (NEXT-4 overlap bands), else c0
+  int32_t halo_bands;             // leading overlap bands (outputs to halo_out), 0 without a halo
+  int32_t export_band;            // the band whose east edge goes to next_edge (nbands-1 without a halo)
+  void* halo_out;                 // overlap bands' scratch plane: rows x halo_pitch int32
+  int64_t halo_pitch;
   int32_t match, mismatch, gap;
   int32_t alphabet;               // SEQCMP: 0 = any byte codes, 1..8 = codes < alphabet
   // tuning

@@ -54,6 +54,7 @@
 namespace wfk {
 
 cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols, int box_rows);
+cudaError_t encode_map_2d(CUtensorMap* m, void* base, int cols, int rows, int64_t pitch_elems, int box_cols, int box_rows);
 
 namespace nw8 {
 
@@ -201,9 +202,10 @@ struct Warp {
   static_assert(SR * ROWB <= 65536, "staging slot arithmetic");
 
   const SweepLaunch& L;
-  const CUtensorMap* tmap;
+  const CUtensorMap* tmap;   // this band's output map: the slab's plane, or (NEXT-4 overlap bands) the scratch plane
   const int band, lane;
   const bool is31;
+  int ocol;                  // this warp's first column in tmap's plane
   int rows;
   int32_t gap, mmatch, mmis;
   int32_t gk[K];          // (m+1) g
@@ -220,13 +222,16 @@ struct Warp {
   uint32_t ring_out;      // shared address of ring WI + 1
   int32_t* gout;          // last warp (WF_NW8_DIRECT_EAST): the next band's / slab's global ring, row r at gout[r]
   bool east_out;          // ... and there is one (not the last band of the last slab); lane 31 only
+  int32_t* gx;            // NEXT-4 halo export band: the next slab's ring as a second destination
+  bool east_x;
   int32_t east_last;      // last warp: lane 31's east word of the current step
   uint32_t x_s;           // shared address of the x copy (x of row r at x_s + r - 1)
   int32_t best = 0, best_row = 0;   // LOCAL: best cell value of the lane and the first row reaching it
   int32_t vrow;           // NW: r c of the lane's first virtual row r = -lane (0 for SW)
 
-  __device__ __forceinline__ Warp(const SweepLaunch& L_, const CUtensorMap* tm, const S& sm, int band_, int lane_)
-      : L(L_), tmap(tm), band(band_), lane(lane_), is31(lane_ == 31) {
+  __device__ __forceinline__ Warp(const SweepLaunch& L_, const CUtensorMap* tm, const CUtensorMap* tm_halo, const S& sm,
+                                  int band_, int lane_)
+      : L(L_), tmap(band_ < L_.halo_bands ? tm_halo : tm), band(band_), lane(lane_), is31(lane_ == 31) {
     rows = L.rows;
     gap = L.gap;
     mmatch = L.match;
@@ -235,8 +240,9 @@ struct Warp {
     for (int m = 0; m < K; ++m) gk[m] = (m + 1) * gap;
     gLx = is31 ? -(1 << 29) : K * gap;
     const uint8_t* y = static_cast<const uint8_t*>(L.col_in);
-    wcol = band * L.band_w + WI * 32 * K;
-    const int jb = L.c0 + wcol + lane * K;   // global 0-based first column of the lane
+    wcol = band * L.band_w + WI * 32 * K;      // relative to the first computed column cc0
+    ocol = band < L.halo_bands ? wcol : wcol - L.halo_bands * L.band_w;
+    const int jb = L.cc0 + wcol + lane * K;   // global 0-based first column of the lane
     // NW: lane l starts at step 1 on row 1 - l.  Instead of predicating every state update of the
     // ramp-up steps (rows <= 0), the row-0 boundary is extended to virtual rows r <= 0 by
     // V(r, j) = j g + r c with c = max(1, g, max(match, mismatch) - g): V is a fixed point of the
@@ -263,12 +269,19 @@ struct Warp {
     ring_out = saddr(sm.ring) + uint32_t(WI + 1) * RR * 4;
     gout = nullptr;
     east_out = false;
+    gx = nullptr;
+    east_x = false;
     if (WF_NW8_DIRECT_EAST && WI == WARPS - 1) {
       int32_t* gbase = reinterpret_cast<int32_t*>(L.edge);
       gout = (band + 1 < L.nbands) ? gbase + size_t(band + 1) * gring_stride(rows) + kGOff
-                                   : (L.next_edge ? reinterpret_cast<int32_t*>(L.next_edge) + kGOff : nullptr);
+                                   : (L.next_edge && band == L.export_band ? reinterpret_cast<int32_t*>(L.next_edge) + kGOff
+                                                                           : nullptr);
+      // NEXT-4 halo: the export band also feeds the next slab (whose overlap starts after it)
+      gx = (band + 1 < L.nbands && band == L.export_band && L.next_edge)
+               ? reinterpret_cast<int32_t*>(L.next_edge) + kGOff : nullptr;
       east_out = gout != nullptr;
       east_out = east_out && is31;
+      east_x = gx != nullptr && is31;
     }
     x_s = saddr(sm.x);
   }
@@ -376,7 +389,10 @@ struct Warp {
         // quad of the next band's / slab's global ring; rows <= 0 or > rows land in its slack,
         // which is never read)
         eq[u & 3] = east_last;
-        if ((u & 3) == 3) stg128_if(east_out, gout + (s0 - 33 + u), make_int4(eq[0], eq[1], eq[2], eq[3]));
+        if ((u & 3) == 3) {
+          stg128_if(east_out, gout + (s0 - 33 + u), make_int4(eq[0], eq[1], eq[2], eq[3]));
+          if (gx != nullptr) stg128_if(east_x, gx + (s0 - 33 + u), make_int4(eq[0], eq[1], eq[2], eq[3]));   // uniform
+        }
       }
     }
   }
@@ -387,7 +403,7 @@ struct Warp {
     __syncwarp();
     if (lane == 0) {
       bulk_wait_read<1>();   // slots of the box issued two publishes ago may be rewritten next
-      tma_store_2d(tmap, stage_s + uint32_t((r0 - 1) & (SR - 1)) * ROWB, wcol, r0 - 1);
+      tma_store_2d(tmap, stage_s + uint32_t((r0 - 1) & (SR - 1)) * ROWB, ocol, r0 - 1);
       bulk_commit();
     }
     __syncwarp();
@@ -517,9 +533,9 @@ struct Helper {
   unsigned nslow = 0;     // WF_TRACE: blocks whose inbound quads were not all there when delivered
   Watchdog wd;
 
-  __device__ __forceinline__ Helper(const SweepLaunch& L_, const CUtensorMap* tm, const S& sm, int band_, int lane_,
-                                    bool first)
-      : L(L_), tmap(tm), band(band_), lane(lane_) {
+  __device__ __forceinline__ Helper(const SweepLaunch& L_, const CUtensorMap* tm, const CUtensorMap* tm_halo, const S& sm,
+                                    int band_, int lane_, bool first)
+      : L(L_), tmap(band_ < L_.halo_bands ? tm_halo : tm), band(band_), lane(lane_) {
     rows = L.rows;
     stage0 = saddr(sm.stage);
     elast = ((rows + 31 + U - 1) / U) * U;
@@ -586,7 +602,7 @@ struct Helper {
       if (e >= 64 && (e & 31) == 0 && e <= elast) {
         const int r0 = e - 63;
         tma_store_2d(tmap, stage0 + uint32_t(w) * SR * S::ROWB + uint32_t((r0 - 1) & (SR - 1)) * S::ROWB,
-                     band * L.band_w + w * 32 * K, r0 - 1);
+                     (band < L.halo_bands ? band : band - L.halo_bands) * L.band_w + w * 32 * K, r0 - 1);
       }
     }
     bulk_commit();
@@ -611,7 +627,7 @@ struct Helper {
     const int Tw = rows + 31;
     const int Tc = Tw + (WARPS - 1) * LAG;
     const int Ll = (WARPS - 1) * LAG;   // the last compute warp's lag
-    if (outbound && band + 1 >= L.nbands && L.next_edge && L.ack_self) {
+    if (band == L.export_band && L.next_edge && L.ack_self) {
       // the next slab must have drained (and reset) this ring in the previous run
       wd.start();
       for (;;) {
@@ -680,24 +696,24 @@ struct Helper {
 };
 
 template <int K, int WARPS, int WI, bool LOCAL, int U>
-__device__ __forceinline__ void dispatch(const SweepLaunch& L, const CUtensorMap* tm, const Smem<K, WARPS>& sm, int band,
-                                         int warp, int lane, bool first) {
+__device__ __forceinline__ void dispatch(const SweepLaunch& L, const CUtensorMap* tm, const CUtensorMap* tmh,
+                                         const Smem<K, WARPS>& sm, int band, int warp, int lane, bool first) {
   if constexpr (WI < WARPS) {
     if (warp == WI) {
       if constexpr (WI == 0) {
         if (first) {
-          Warp<K, WARPS, 0, true, LOCAL, U> w(L, tm, sm, band, lane);
+          Warp<K, WARPS, 0, true, LOCAL, U> w(L, tm, tmh, sm, band, lane);
           w.run();
           return;
         }
       }
-      Warp<K, WARPS, WI, false, LOCAL, U> w(L, tm, sm, band, lane);
+      Warp<K, WARPS, WI, false, LOCAL, U> w(L, tm, tmh, sm, band, lane);
       w.run();
     } else {
-      dispatch<K, WARPS, WI + 1, LOCAL, U>(L, tm, sm, band, warp, lane, first);
+      dispatch<K, WARPS, WI + 1, LOCAL, U>(L, tm, tmh, sm, band, warp, lane, first);
     }
   } else {
-    Helper<K, WARPS, LOCAL, U> h(L, tm, sm, band, lane, first);
+    Helper<K, WARPS, LOCAL, U> h(L, tm, tmh, sm, band, lane, first);
     if (WF_NW8_HELPER_TMA == 2 && warp == WARPS + 1) h.run_storer();
     else h.run();
   }
@@ -705,7 +721,8 @@ __device__ __forceinline__ void dispatch(const SweepLaunch& L, const CUtensorMap
 
 template <int K, int WARPS, bool LOCAL, int U>
 __global__ void __launch_bounds__((WARPS + kExtraWarps) * 32, 1)
-    nw8_kernel(const __grid_constant__ SweepLaunch L, const __grid_constant__ CUtensorMap tmap) {
+    nw8_kernel(const __grid_constant__ SweepLaunch L, const __grid_constant__ CUtensorMap tmap,
+               const __grid_constant__ CUtensorMap tmap_halo) {
   using S = Smem<K, WARPS>;
   extern __shared__ __align__(16) unsigned char nw8_smem_raw[];
   const S sm(nw8_smem_raw);
@@ -726,7 +743,7 @@ __global__ void __launch_bounds__((WARPS + kExtraWarps) * 32, 1)
   }
   for (int band = blockIdx.x; band < L.nbands; band += gridDim.x) {
     __syncthreads();
-    dispatch<K, WARPS, 0, LOCAL, U>(L, &tmap, sm, band, warp, lane, L.first_slab && band == 0);
+    dispatch<K, WARPS, 0, LOCAL, U>(L, &tmap, &tmap_halo, sm, band, warp, lane, L.first_slab && band == 0);
     __syncthreads();
     if (run_failed(L)) return;
   }
@@ -736,13 +753,18 @@ constexpr int kU = WF_NW8_U;   // steps per lockstep block
 
 template <int K, int WARPS, int U>
 cudaError_t launch(const SweepLaunch& L, cudaStream_t s, size_t smem) {
-  CUtensorMap tmap;
+  CUtensorMap tmap, tmap_halo;
   cudaError_t e = encode_plane_map(&tmap, L, 32 * K, 32);
   if (e != cudaSuccess) return e;
+  tmap_halo = tmap;
+  if (L.halo_bands > 0) {   // NEXT-4 overlap bands: their own scratch plane
+    e = encode_map_2d(&tmap_halo, L.halo_out, int(L.halo_pitch), L.rows, L.halo_pitch, 32 * K, 32);
+    if (e != cudaSuccess) return e;
+  }
   auto kfn = L.local ? nw8_kernel<K, WARPS, true, U> : nw8_kernel<K, WARPS, false, U>;
   e = cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
-  kfn<<<L.grid, (WARPS + kExtraWarps) * 32, smem, s>>>(L, tmap);
+  kfn<<<L.grid, (WARPS + kExtraWarps) * 32, smem, s>>>(L, tmap, tmap_halo);
   return cudaGetLastError();
 }
 

@@ -79,6 +79,16 @@ cudaError_t encode_plane_map_f(CUtensorMap* m, const SweepLaunch& L, int plane, 
                    CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   return r == CUDA_SUCCESS ? cudaSuccess : cudaErrorInvalidValue;
 }
+// int32 [rows][cols] plane at `base` with a row pitch of pitch_elems elements
+cudaError_t encode_map_2d(CUtensorMap* m, void* base, int cols, int rows, int64_t pitch_elems, int box_cols, int box_rows) {
+  SweepLaunch L{};
+  L.c0 = 0;
+  L.c1 = cols;
+  L.rows = rows;
+  L.pitch = pitch_elems;
+  L.out[0] = base;
+  return encode_plane_map_f(m, L, 0, box_cols, box_rows);
+}
 cudaError_t encode_plane_map(CUtensorMap* m, const SweepLaunch& L, int box_cols, int box_rows) {
   return encode_plane_map_f(m, L, 0, box_cols, box_rows);
 }

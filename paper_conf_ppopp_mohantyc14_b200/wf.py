@@ -41,7 +41,7 @@ class Layout:
 
 def make_params(fn, dim, *, cols=0, tsize=0, dsize=0, lane_cols=0, warps=0, skew=0, strip=0, ngpus=1,
                 match=0, mismatch=0, gap=0, local=0, transport="p2p", max_ctas=0, watchdog_cycles=0,
-                alphabet=0, kernel=0) -> WfParams:
+                alphabet=0, kernel=0, halo=0) -> WfParams:
     p = WfParams()
     p.dim = int(dim)
     p.cols = int(cols)
@@ -60,6 +60,7 @@ def make_params(fn, dim, *, cols=0, tsize=0, dsize=0, lane_cols=0, warps=0, skew
     p.watchdog_cycles = int(watchdog_cycles)
     p.alphabet = int(alphabet)
     p.kernel = int(kernel)
+    p.halo = int(halo)
     return p
 
 

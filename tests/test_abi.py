@@ -102,7 +102,7 @@ def test_strip_axis():
 
 def test_reserved_fields_must_be_zero():
     p = make_params("seqcmp", 64)
-    p.reserved[2] = 1
+    p.reserved[1] = 1
     lay = _abi.WfLayout()
     st = _abi.lib().wf_query(ctypes.byref(p), 0, ctypes.byref(lay))
     assert st == _abi.WF_EINVAL and b"reserved" in _abi.lib().wf_last_error(None)
@@ -177,3 +177,21 @@ def test_create_without_dist_rejects_multi_slab():
     ctx = ctypes.c_void_p()
     st = _abi.lib().wf_create(ctypes.byref(p), None, ctypes.byref(ctx))
     assert st == _abi.WF_EINVAL and not ctx.value
+
+
+def test_halo_overlap_validation():
+    """NEXT-4 halo (include/wf.h wf_params.halo): whole bands of the generation-8 NW sweep,
+    multi-slab only; slab g > 0 computes halo more columns but outputs the same ones."""
+    base = query("seqcmp", 4096, rank=1, ngpus=2)
+    lay = query("seqcmp", 4096, rank=1, ngpus=2, halo=base.band_cols)
+    assert (lay.col_begin, lay.col_end) == (base.col_begin, base.col_end)
+    assert lay.nbands == base.nbands + 1
+    assert query("seqcmp", 4096, rank=0, ngpus=2, halo=base.band_cols).nbands == base.nbands
+    for kw, st in ((dict(halo=100), _abi.WF_EINVAL), (dict(halo=-256), _abi.WF_EINVAL),
+                   (dict(halo=256, ngpus=1), _abi.WF_EINVAL), (dict(halo=256, local=1), _abi.WF_EUNSUPPORTED),
+                   (dict(halo=256, kernel=4), _abi.WF_EUNSUPPORTED), (dict(halo=256 * 8), _abi.WF_EINVAL)):
+        kw.setdefault("ngpus", 2)
+        e = _err("seqcmp", 4096, **kw)
+        assert e.status == st and "halo" in str(e), (kw, e)
+    e = _err("synthetic", 4096, tsize=10, dsize=1, ngpus=2, halo=32)
+    assert e.status == _abi.WF_EUNSUPPORTED

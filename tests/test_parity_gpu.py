@@ -83,6 +83,23 @@ def test_seqcmp_strips_local_slabs(strip, G):
     assert np.array_equal(H, g)
 
 
+@pytest.mark.parametrize("G,halo,dim", [(2, 256, 1100), (2, 256, 3001), (3, 256, 3001), (2, 512, 3001), (4, 256, 4097)])
+def test_seqcmp_halo_overlap_slabs(G, halo, dim):
+    """NEXT-4 (wf_params.halo): slab g > 0 recomputes halo columns of slab g-1 into a scratch plane
+    and takes its west input from slab g-1's column c0 - halo - 1; the grid is unchanged."""
+    H, g = _seq(dim, ngpus=G, halo=halo, seed=(dim + 3, dim + 4), alphabet=4)
+    assert np.array_equal(H, g)
+
+
+@pytest.mark.parametrize("halo", [256, 512])
+def test_seqcmp_halo_reruns_and_scoring(halo):
+    x, y = workloads.seqcmp_inputs(2500, 2500, seed_x=11, seed_y=12)
+    H = oracle.seqcmp(x, y, 2, -3, -2)
+    for _ in range(2):
+        (g,) = run_gpu("seqcmp", 2500, (x, y), ngpus=2, halo=halo, match=2, mismatch=-3, gap=-2)
+        assert np.array_equal(H, g)
+
+
 @pytest.mark.parametrize("k,w,d", [(4, 2, 1), (2, 4, 1), (4, 1, 2)])
 @pytest.mark.parametrize("dim", [33, 777, 1100])
 def test_seqcmp_generation4_kernel(k, w, d, dim):

@@ -141,7 +141,7 @@ def compiled(cfg, k, w, d, impl, strip=0):
     return (lay.lane_cols, lay.warps, lay.skew) == (k, w, d)
 
 
-def time_slabs(cfg, k, w, d, impl, host, G, reps, strip=0):
+def time_slabs(cfg, k, w, d, impl, host, G, reps, strip=0, **extra):
     """G column slabs of the same grid linked by the per-row P2P hand-off.  Virtual slabs (one
     GPU): device time between two events on the current stream, which gates every slab stream --
     a ~10 ms device-side sleep ahead of the start event holds the slabs back until the host has
@@ -149,7 +149,7 @@ def time_slabs(cfg, k, w, d, impl, host, G, reps, strip=0):
     ngpu = torch.cuda.device_count()
     devices = [g % ngpu for g in range(G)]
     ls = LocalSlabs(cfg.fn, cfg.dim, G, devices=devices, lane_cols=k, warps=w, skew=d, kernel=impl, strip=strip,
-                    **fn_kw(cfg))
+                    **fn_kw(cfg), **extra)
     virtual = len(set(devices)) == 1
     try:
         per = [inputs_for(cfg.fn, cfg.dim, cfg.dsize, torch.device("cuda", s.device))[1] for s in ls.slabs]
