@@ -397,6 +397,15 @@ struct SynWarp {
 __host__ __device__ constexpr unsigned syn_feed_ns(int ds) {
   return WF_SYN_FEED_NS >= 0 ? unsigned(WF_SYN_FEED_NS) : (ds <= 2 ? 0u : 64u);
 }
+#ifndef WF_SYN_DISCARD
+// 1: the feeder drops each fully consumed 128-byte line of its band's inbound LL ring from L2
+// without write-back (discard.global.L2): the words are dead once copied to shared memory, so the
+// ring costs no DRAM traffic (C5a: 1.106x -> ~1.0x algorithmic, profiles/ncu_traffic.json)
+#define WF_SYN_DISCARD 1
+#endif
+__device__ __forceinline__ void discard_l2_line(const void* p) {
+  asm volatile("discard.global.L2 [%0], 128;" ::"l"(p) : "memory");
+}
 template <int DS, int K, int WARPS, int NPW = 1>
 __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS>& pol, const SynSmem<DS, K, WARPS>& sm,
                                            int band, int lane) {
@@ -405,6 +414,9 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
   const int rows = L.rows;
   const bool boundary = L.first_slab && band == 0;
   const unsigned long long* src = L.edge + size_t(band) * edge_stride(rows) * NF;
+  // next ring line to discard: the first 128-byte line that starts at or after row 1's words (a
+  // line below it may hold the previous band's ring, which another feeder still reads)
+  uintptr_t disc = (reinterpret_cast<uintptr_t>(src + size_t(1) * NF) + 127) & ~uintptr_t(127);
   int feed = 1, seen = 0;
   Watchdog wd;
   wd.start();
@@ -452,6 +464,14 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
       __threadfence_block();
       feed += n;
       if (lane == 0) sts_vol_i(sm.wprog + 0, feed - 1);
+      if (WF_SYN_DISCARD && !boundary) {
+        // every line wholly below the consumed frontier (rows < feed), one line per lane
+        const uintptr_t end = reinterpret_cast<uintptr_t>(src + size_t(feed) * NF) & ~uintptr_t(127);
+        const uintptr_t a = disc + uintptr_t(lane) * 128;
+        if (a < end) discard_l2_line(reinterpret_cast<const void*>(a));
+        const uintptr_t nd = disc + 32 * 128;
+        disc = end > disc ? (end < nd ? end : nd) : disc;
+      }
       wd.start();
       if (feed > rows && !L.first_slab && band == 0 && L.ack_prev) {
         __syncwarp();
