@@ -525,3 +525,25 @@ def test_nash_c3_prefix():
     _check_nash(o, g, rows=48)
     cnt, first = g[0], g[1]
     assert np.all((first == -1) == (cnt == 0)) and cnt.max() <= 16 * 16
+
+
+# ---- transport = "nccl" in one process (the message moved by a device copy instead of send/recv)
+@pytest.mark.parametrize("case", ["nw8_staged", "syn_staged"])
+def test_staged_transport_in_process(case):
+    import sys
+    import os
+    sys.path.insert(0, os.path.join(os.path.dirname(os.path.dirname(os.path.abspath(__file__))), "tools"))
+    import sanitize_cases
+    sanitize_cases.run(case)
+
+
+@pytest.mark.parametrize("G", [2, 3])
+def test_staged_transport_in_process_nw_three_slabs(G):
+    import sys
+    import os
+    sys.path.insert(0, os.path.join(os.path.dirname(os.path.dirname(os.path.abspath(__file__))), "tools"))
+    from sanitize_cases import run_staged_in_process
+    x, y = workloads.seqcmp_inputs(1500, 1500, seed_x=21, seed_y=22)
+    H = oracle.seqcmp(x, y, 1, -1, -1)
+    (g,) = run_staged_in_process("seqcmp", 1500, (x, y), ngpus=G, transport="nccl", alphabet=4)
+    assert np.array_equal(g, H)

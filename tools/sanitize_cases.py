@@ -37,7 +37,39 @@ CASES = {
     "syn_generic": ("synthetic", 150, {"tsize": 5, "dsize": 2, "kernel": 4}),
     "syn_slabs2": ("synthetic", 150, {"tsize": 3, "dsize": 2, "ngpus": 2}),
     "nash": ("nash", 40, {"tsize": 16, "dsize": 4}),
+    "nw8_halo": ("seqcmp", 1100, {"ngpus": 2, "halo": 256}),
+    "nw8_staged": ("seqcmp", 600, {"ngpus": 2, "transport": "nccl"}),
+    "syn_staged": ("synthetic", 150, {"tsize": 3, "dsize": 2, "ngpus": 2, "transport": "nccl"}),
 }
+
+
+def run_staged_in_process(fn, dim, inputs, **kw):
+    """transport="nccl" slabs in ONE process: each slab's edge message is exported into a device
+    buffer and imported by its successor (the copy the process group's send/recv makes between
+    ranks), slabs run in order; returns the concatenated planes."""
+    import torch
+    from _gpu_helpers import dev_inputs
+    from paper_conf_ppopp_mohantyc14_b200.wf import Wavefront
+    G = kw.pop("ngpus")
+    dev = torch.device("cuda", torch.cuda.current_device())
+    slabs = [Wavefront(fn, dim, rank=g, device=dev.index, ngpus=G, **kw) for g in range(G)]
+    try:
+        args = dev_inputs(fn, inputs, dev)
+        outs, msg = [], None
+        for g, w in enumerate(slabs):
+            if g > 0:
+                w.edge_import(msg)
+            outs.append(w.run(*args))
+            if g < G - 1:
+                msg = torch.empty(w.edge_bytes(), dtype=torch.uint8, device=dev)
+                w.edge_export(msg)
+        torch.cuda.synchronize()
+        for w in slabs:
+            w.sync()
+        return [np.concatenate([o[f].cpu().numpy() for o in outs], axis=1) for f in range(len(outs[0]))]
+    finally:
+        for w in slabs:
+            w.close()
 
 
 def run(name):
@@ -46,20 +78,21 @@ def run(name):
     from _gpu_helpers import run_gpu
     fn, dim, kw = CASES[name]
     kw = dict(kw)
+    runner = run_staged_in_process if kw.get("transport") == "nccl" else run_gpu
     if fn == "seqcmp":
         x, y = workloads.seqcmp_inputs(dim)
         want = [oracle.seqcmp(x, y, 1, -1, -1, local=bool(kw.get("local", 0)))]
-        got = run_gpu(fn, dim, (x, y), **kw)
+        got = runner(fn, dim, (x, y), **kw)
     elif fn == "synthetic":
         u, v, top, left = workloads.synthetic_inputs(dim, dim, kw["dsize"])
         i0, i1, f = oracle.synthetic(u, v, top, left, kw["tsize"])
         want = [i0, i1] + [f[d] for d in range(f.shape[0])]
-        got = run_gpu(fn, dim, (u, v, top, left), **kw)
+        got = runner(fn, dim, (u, v, top, left), **kw)
     else:
         r, c, top, left = workloads.nash_inputs(dim, dim)
         o = oracle.nash(r, c, top, left, nstrat=kw["tsize"])
         want = [o[p] for p in range(4)]
-        got = run_gpu(fn, dim, (r, c, top, left), **kw)
+        got = runner(fn, dim, (r, c, top, left), **kw)
     for p, (g, o) in enumerate(zip(got, want)):
         o = np.asarray(o)
         g = np.asarray(g).view(o.dtype)
