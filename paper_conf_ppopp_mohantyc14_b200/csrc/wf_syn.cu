@@ -226,11 +226,15 @@ struct SynWarp {
     }
   }
 
-  // lane 0's west words + row input of row r (all lanes load: broadcast)
+  // lane 0's west words + row input of row r (all lanes load: broadcast).  Plain loads: every
+  // block starts after wait_ctr observed the producer's counter covering the block's rows and
+  // fenced (__threadfence_block, also a compiler barrier), so the words are there and no load
+  // can move above it; unlike volatile loads they need not stay in program order with the
+  // step's shared stores (C5a 4.044 -> 3.876 ms, profiles/r02_syn_lds_ab.txt)
   __device__ __forceinline__ void issue(int r, uint32_t (&w)[NWD]) const {
     const uint32_t* p = sm.slot(warp, r);
 #pragma unroll
-    for (int i = 0; i < NWD; ++i) w[i] = (i == NF || use(i)) ? lds_vol_u32(p + i) : 0u;
+    for (int i = 0; i < NWD; ++i) w[i] = (i == NF || use(i)) ? p[i] : 0u;
   }
   // wait until a shared progress counter reaches `need` (seen caches the last value)
   __device__ __forceinline__ bool wait_ctr(const int* ctr, int need, int& seen) {
