@@ -81,6 +81,16 @@ struct SynSmem {
   }
 };
 
+#ifndef WF_SYN_STEP_WAIT
+// Heavy cells (tsize x dsize >= 1000, UB = 4): a compute warp waits for its west words row by row
+// (a cached copy of the producer's counter, re-read only when it does not cover the step's row)
+// instead of for the whole UB-row block, so the band-to-band lag loses up to UB - 1 steps
+// (C5c 78.28 -> 76.19 ms).  Light cells keep the block wait: there a step is short and the
+// per-step check at the producer's heels costs more than it saves (C5a 3.88 -> 5.55 ms); so do
+// many-plane heavy cells (C5d 129.6 -> 131.8 ms with it); profiles/r02_syn_lds_ab.txt.
+// 0 = never, 1 = heavy cells with dsize <= 2, 2 = always (experiments).
+#define WF_SYN_STEP_WAIT 1
+#endif
 __device__ __forceinline__ void sts_u32_pred(bool p, uint32_t* a, uint32_t v) {
   asm volatile("{ .reg .pred q; setp.ne.b32 q, %2, 0; @q st.volatile.shared.u32 [%0], %1; }" ::"r"(
                    static_cast<uint32_t>(__cvta_generic_to_shared(a))),
@@ -250,9 +260,11 @@ struct SynWarp {
     }
   }
 
+  static constexpr bool kStepWait = WF_SYN_STEP_WAIT == 2 || (WF_SYN_STEP_WAIT == 1 && syn_ub(TS, DS) <= 4 && DS <= 2);
+
   template <bool EDGE, bool LAST>
-  __device__ __forceinline__ void block(int t0, uint32_t (&pre)[NWD], uint32_t (&q)[NF], uint32_t& qx,
-                                        unsigned long long* gdst, bool to_peer) {
+  __device__ __forceinline__ bool block(int t0, uint32_t (&pre)[NWD], uint32_t (&q)[NF], uint32_t& qx,
+                                        unsigned long long* gdst, bool to_peer, int& seen_w) {
     uint32_t* nring = LAST ? nullptr : sm.ll + size_t(warp + 1) * kSynLL * NWD;
     const bool glob = LAST && gdst != nullptr;
 #pragma unroll
@@ -263,6 +275,9 @@ struct SynWarp {
 #pragma unroll
       for (int f = 0; f < NF; ++f) Win[f] = (lane == 0) ? pre[f] : q[f];
       const uint32_t xr = (lane == 0) ? pre[NF] : qx;
+      if (kStepWait && u > 0 && t + 2 <= rows && seen_w < t + 2) {   // (u = 0: run() waited)
+        if (!wait_ctr(sm.wprog + warp, t + 2, seen_w)) return false;
+      }
       if (!EDGE || t + 2 <= rows) issue(t + 2, pre);   // next step's words: latency hides behind the cell
       bool active = true;
       if constexpr (EDGE) active = row >= 1 && row <= rows;
@@ -302,6 +317,7 @@ struct SynWarp {
       for (int f = 0; f < NF; ++f) q[f] = use(f) ? __shfl_up_sync(0xffffffffu, Np[K - 1][f], 1) : 0u;
       qx = __shfl_up_sync(0xffffffffu, xr, 1);
     }
+    return true;
   }
 
   __device__ __forceinline__ bool run() {
@@ -335,7 +351,7 @@ struct SynWarp {
     static_assert(U % UB == 0, "hand-off blocks tile the write-back window");
     for (int t0 = 0; t0 < T; t0 += UB) {
       // this block reads rows t0+2 .. t0+UB+1 of my ring (row t0+1 is already in pre)
-      if (!wait_ctr(sm.wprog + warp, min(t0 + UB + 1, rows), seen_w)) return false;
+      if (!wait_ctr(sm.wprog + warp, min(kStepWait ? t0 + 2 : t0 + UB + 1, rows), seen_w)) return false;
       if (lane == 0) sts_vol_i(sm.rprog + warp + kRd, t0 + 1);   // rows <= t0+1 of my ring consumed
       // lane 31 writes rows t0-30 .. t0-31+UB into the next ring: their slots must be free
       if (!last && !wait_ctr(sm.rprog + warp + 1, t0 - 31 + UB - kSynLL, seen_r)) return false;
@@ -344,13 +360,15 @@ struct SynWarp {
         __syncwarp();
       }
       const bool steady = t0 >= 32 && t0 + UB + 1 <= rows;
+      bool ok;
       if (last) {
-        if (steady) block<false, true>(t0, pre, q, qx, gdst, to_peer);
-        else block<true, true>(t0, pre, q, qx, gdst, to_peer);
+        if (steady) ok = block<false, true>(t0, pre, q, qx, gdst, to_peer, seen_w);
+        else ok = block<true, true>(t0, pre, q, qx, gdst, to_peer, seen_w);
       } else {
-        if (steady) block<false, false>(t0, pre, q, qx, gdst, to_peer);
-        else block<true, false>(t0, pre, q, qx, gdst, to_peer);
+        if (steady) ok = block<false, false>(t0, pre, q, qx, gdst, to_peer, seen_w);
+        else ok = block<true, false>(t0, pre, q, qx, gdst, to_peer, seen_w);
       }
+      if (!ok) return false;
       wf_jitter(15);
       // publish lane 31's rows of the block to the next warp (one fence per block)
       const int r31_last = min(t0 + UB - 31, rows);

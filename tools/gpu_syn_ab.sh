@@ -7,3 +7,5 @@ done
 unset WF_TEST_LIB
 timeout 900 python tools/ab_time.py --config C5a --rounds 4 "$@" > gpurun_out/synab_c5a.txt 2>&1
 timeout 900 python tools/ab_time.py --config C2 --rounds 3 "$@" > gpurun_out/synab_c2.txt 2>&1
+timeout 900 python tools/ab_time.py --config C5c --rounds 2 "$@" > gpurun_out/synab_c5c.txt 2>&1
+timeout 900 python tools/ab_time.py --config C5b --rounds 3 "$@" > gpurun_out/synab_c5b.txt 2>&1
