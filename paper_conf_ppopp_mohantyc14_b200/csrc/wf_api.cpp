@@ -366,7 +366,9 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
 
   // per band: the inbound LL ring (edge_stride rows) plus 32 slots of slack on each side (the
   // generation-8 ring is addressed at +32 so that ramp-up / drain rows never leave it)
-  c->edge_bytes = (size_t)pl.nbands * (wfk::edge_stride(p->dim) + 64) * pl.nf * sizeof(unsigned long long);
+  // synthetic rings hold row records padded to 4-word multiples (wf_syn.cu syn_ring_words)
+  const int ring_words = p->fn == WF_FN_SYNTHETIC ? ((pl.nf + 3) & ~3) : pl.nf;
+  c->edge_bytes = (size_t)pl.nbands * (wfk::edge_stride(p->dim) + 64) * ring_words * sizeof(unsigned long long);
   e = cudaMalloc(&c->base, kCtrlBytes + c->edge_bytes);
   // control block 0; edge rings 0x80 bytes: the generation-8 EMPTY word (0x80808080), and a tag
   // no epoch ever takes for the LL-word generations
@@ -379,7 +381,7 @@ wf_status wf_create(const wf_params* p, const wf_dist* dist, wf_ctx** out) {
   // transport NCCL: the last band stores its east edge into a local outbound ring (same layout as
   // a band-0 inbound ring) which the caller ships with send/recv (wf_edge_export / import)
   c->staged = p->transport == WF_TRANSPORT_NCCL && c->world > 1;
-  c->stage_bytes = (wfk::edge_stride(p->dim) + 64) * pl.nf * sizeof(unsigned long long);
+  c->stage_bytes = (wfk::edge_stride(p->dim) + 64) * ring_words * sizeof(unsigned long long);
   if (e == cudaSuccess && c->staged && c->rank < c->world - 1) {
     e = cudaMalloc(&c->stage, c->stage_bytes);
     if (e == cudaSuccess) e = cudaMemset(c->stage, 0x80, c->stage_bytes);

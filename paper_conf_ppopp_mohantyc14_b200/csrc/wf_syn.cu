@@ -51,9 +51,17 @@ struct SynMaps {
   CUtensorMap m[WF_MAX_PLANES];
 };
 
+// Global LL ring record of a row: NF 8-byte words (value | run-epoch tag) padded to a multiple
+// of 4 words, so the band's last lane writes each row with 32-byte stores that cover whole L2
+// sectors (no fill read of the sector; the consumer discards consumed lines, so the ring costs
+// no DRAM traffic -- profiles/r02_c5a_traffic.txt).  The host sizes the rings with the same
+// padding (wf_api.cpp: ring_words).
+__host__ __device__ constexpr int syn_ring_words(int nf) { return (nf + 3) & ~3; }
+
 template <int DS, int K, int WARPS>
 struct SynSmem {
   static constexpr int NF = 2 + DS;         // output planes / west words per row
+  static constexpr int NFP = syn_ring_words(NF);   // global ring words per row
   static constexpr int NWD = NF + 1;        // + the row input u_i
   static constexpr int U = syn_ut(DS);
   // staging rows alive: skew 31 + the TMA window being filled + the window whose TMA store
@@ -104,6 +112,13 @@ __device__ __forceinline__ uint32_t lds_vol_u32(const uint32_t* p) { return *rei
 __device__ __forceinline__ void stg_sys_u64_pred(bool p, unsigned long long* a, unsigned long long v) {
   asm volatile("{ .reg .pred q; setp.ne.b32 q, %2, 0; @q st.relaxed.sys.global.u64 [%0], %1; }" ::"l"(a), "l"(v),
                "r"(static_cast<int>(p))
+               : "memory");
+}
+// 32-byte strong store of 4 LL words (STG.E.ENL2.256): whole L2 sectors
+__device__ __forceinline__ void stg_sys_v4_pred(bool p, unsigned long long* a, unsigned long long w0, unsigned long long w1,
+                                                unsigned long long w2, unsigned long long w3) {
+  asm volatile("{ .reg .pred q; setp.ne.b32 q, %5, 0; @q st.relaxed.sys.global.v4.b64 [%0], {%1, %2, %3, %4}; }" ::"l"(a),
+               "l"(w0), "l"(w1), "l"(w2), "l"(w3), "r"(static_cast<int>(p))
                : "memory");
 }
 __device__ __forceinline__ void stg_gpu_u64_pred(bool p, unsigned long long* a, unsigned long long v) {
@@ -307,11 +322,21 @@ struct SynWarp {
       } else {
         // system scope: the next slab's ring may be a peer (NVLink) mapping; measured no slower
         // than gpu scope for the next band's ring on the same GPU
-        unsigned long long* g = gdst + size_t(row) * NF;
+        unsigned long long* g = gdst + size_t(row) * S::NFP;
         (void)to_peer;
+        if constexpr (PW < 0) {   // the whole record: 32-byte stores (full L2 sectors)
+          const uint32_t ep = L.epoch;
 #pragma unroll
-        for (int f = 0; f < NF; ++f)
-          if (use(f)) stg_sys_u64_pred(pub && glob, g + f, ll_pack(Np[K - 1][f], L.epoch));
+          for (int c = 0; c < S::NFP; c += 4)
+            stg_sys_v4_pred(pub && glob, g + c, ll_pack(c < NF ? Np[K - 1][c] : 0u, ep),
+                            ll_pack(c + 1 < NF ? Np[K - 1][c + 1 < NF ? c + 1 : 0] : 0u, ep),
+                            ll_pack(c + 2 < NF ? Np[K - 1][c + 2 < NF ? c + 2 : 0] : 0u, ep),
+                            ll_pack(c + 3 < NF ? Np[K - 1][c + 3 < NF ? c + 3 : 0] : 0u, ep));
+        } else {   // plane-split warps own some fields of the record
+#pragma unroll
+          for (int f = 0; f < NF; ++f)
+            if (use(f)) stg_sys_u64_pred(pub && glob, g + f, ll_pack(Np[K - 1][f], L.epoch));
+        }
       }
 #pragma unroll
       for (int f = 0; f < NF; ++f) q[f] = use(f) ? __shfl_up_sync(0xffffffffu, Np[K - 1][f], 1) : 0u;
@@ -333,7 +358,7 @@ struct SynWarp {
       }
     }
     unsigned long long* gdst = nullptr;
-    if (last) gdst = (band + 1 < L.nbands) ? L.edge + size_t(band + 1) * edge_stride(rows) * NF : L.next_edge;
+    if (last) gdst = (band + 1 < L.nbands) ? L.edge + size_t(band + 1) * edge_stride(rows) * S::NFP : L.next_edge;
     const bool to_peer = band + 1 >= L.nbands;
     int seen_w = 0, seen_r = 0;
     uint32_t pre[NWD];
@@ -435,10 +460,11 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
   constexpr int NF = S::NF;
   const int rows = L.rows;
   const bool boundary = L.first_slab && band == 0;
-  const unsigned long long* src = L.edge + size_t(band) * edge_stride(rows) * NF;
+  constexpr int NFP = S::NFP;
+  const unsigned long long* src = L.edge + size_t(band) * edge_stride(rows) * NFP;
   // next ring line to discard: the first 128-byte line that starts at or after row 1's words (a
   // line below it may hold the previous band's ring, which another feeder still reads)
-  uintptr_t disc = (reinterpret_cast<uintptr_t>(src + size_t(1) * NF) + 127) & ~uintptr_t(127);
+  uintptr_t disc = (reinterpret_cast<uintptr_t>(src + size_t(1) * NFP) + 127) & ~uintptr_t(127);
   int feed = 1, seen = 0;
   Watchdog wd;
   wd.start();
@@ -466,7 +492,7 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
       } else {
 #pragma unroll
         for (int f = 0; f < NF; ++f) {
-          const unsigned long long w = ld_relaxed_sys(src + size_t(r) * NF + f);
+          const unsigned long long w = ld_relaxed_sys(src + size_t(r) * NFP + f);
           v[f] = static_cast<uint32_t>(w);
           ok = ok && static_cast<uint32_t>(w >> 32) == L.epoch;
         }
@@ -488,7 +514,7 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
       if (lane == 0) sts_vol_i(sm.wprog + 0, feed - 1);
       if (WF_SYN_DISCARD && !boundary) {
         // every line wholly below the consumed frontier (rows < feed), one line per lane
-        const uintptr_t end = reinterpret_cast<uintptr_t>(src + size_t(feed) * NF) & ~uintptr_t(127);
+        const uintptr_t end = reinterpret_cast<uintptr_t>(src + size_t(feed) * NFP) & ~uintptr_t(127);
         const uintptr_t a = disc + uintptr_t(lane) * 128;
         if (a < end) discard_l2_line(reinterpret_cast<const void*>(a));
         const uintptr_t nd = disc + 32 * 128;
