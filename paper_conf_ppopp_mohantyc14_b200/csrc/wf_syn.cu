@@ -444,6 +444,20 @@ struct SynWarp {
 __host__ __device__ constexpr unsigned syn_feed_ns(int ds) {
   return WF_SYN_FEED_NS >= 0 ? unsigned(WF_SYN_FEED_NS) : (ds <= 2 ? 0u : 64u);
 }
+#ifndef WF_SYN_FEED_WIN
+// How the feeder polls its band's ring (profiles/r02_c5a_traffic.txt, same-box A/Bs):
+//   0 = one 8-byte load per LL word, 32 rows per poll (C5a: fastest, 3.652 ms);
+//   2 = 32-byte loads per record, 32 rows (C5b 7.455 -> 7.288 ms; C5a 3.788 ms);
+//   1 = 32-byte loads and an adaptive window (rows delivered last time + 8, at most 32): fewer
+//       polls of not-yet-written rows (C5a reads 267 -> 160 MB) but C5a 3.695 -> 3.876 ms.
+//  -1 (default) = 2 for 8-word records (dsize >= 3), 0 otherwise.
+#define WF_SYN_FEED_WIN -1
+#endif
+__device__ __forceinline__ void ldg_sys_v4(const unsigned long long* a, unsigned long long (&w)[4]) {
+  asm volatile("ld.relaxed.sys.global.v4.b64 {%0, %1, %2, %3}, [%4];" : "=l"(w[0]), "=l"(w[1]), "=l"(w[2]), "=l"(w[3])
+               : "l"(a)
+               : "memory");
+}
 #ifndef WF_SYN_DISCARD
 // 1: the feeder drops each fully consumed 128-byte line of its band's inbound LL ring from L2
 // without write-back (discard.global.L2): the words are dead once copied to shared memory, so the
@@ -466,6 +480,8 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
   // line below it may hold the previous band's ring, which another feeder still reads)
   uintptr_t disc = (reinterpret_cast<uintptr_t>(src + size_t(1) * NFP) + 127) & ~uintptr_t(127);
   int feed = 1, seen = 0;
+  constexpr int kFeed = WF_SYN_FEED_WIN >= 0 ? WF_SYN_FEED_WIN : (NFP >= 8 ? 2 : 0);
+  int win = 32;   // rows polled (kFeed 1)
   Watchdog wd;
   wd.start();
   while (feed <= rows) {
@@ -489,6 +505,22 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
       xr = pol.row_in(r);
       if (boundary) {
         pol.left(r, v);
+      } else if (kFeed) {
+        if (lane < win) {
+#pragma unroll
+          for (int c = 0; c < NFP; c += 4) {
+            unsigned long long w[4];
+            ldg_sys_v4(src + size_t(r) * NFP + c, w);
+#pragma unroll
+            for (int k = 0; k < 4; ++k)
+              if (c + k < NF) {
+                v[c + k] = static_cast<uint32_t>(w[k]);
+                ok = ok && static_cast<uint32_t>(w[k] >> 32) == L.epoch;
+              }
+          }
+        } else {
+          ok = false;
+        }
       } else {
 #pragma unroll
         for (int f = 0; f < NF; ++f) {
@@ -500,6 +532,7 @@ __device__ __forceinline__ bool syn_feeder(const SweepLaunch& L, const PolSyn<DS
     }
     const unsigned m = __ballot_sync(0xffffffffu, ok);
     int n = (m == 0xffffffffu) ? 32 : __ffs(~m) - 1;
+    if (kFeed == 1) win = min(32, max(8, n + 8));
     if (feed + n > rows + 1) n = rows + 1 - feed;
     if (n > 0) {
       if (lane < n) {
