@@ -182,6 +182,15 @@ wf_status validate(const wf_params* p, int rank, Plan* out, wf_ctx* c) {
   }
   defaults(*p, &pl.k, &pl.warps, &pl.skew, &pl.impl);
   pl.strip = p->strip;
+  // small NW grids (at most 3 default bands): 2 compute warps of K = 4 with 8-row strips halve the
+  // in-CTA warp hops that dominate a short sweep -- C1 (dim 512): 0.0558 vs 0.0623 ms; from
+  // dim 1024 up the tilings are within 1 % and (2, 4) wins at C4 (profiles/autotune_C1.json)
+  if (p->fn == WF_FN_SEQCMP && !p->local && !p->lane_cols && !p->warps && !p->skew && !p->strip &&
+      (p->kernel == 0 || p->kernel == 8) && cols <= 768) {
+    pl.k = 4;
+    pl.warps = 2;
+    pl.strip = 8;
+  }
   if (pl.k != 1 && pl.k != 2 && pl.k != 4 && pl.k != 8) return fail(c, WF_EINVAL, "lane_cols=%d not in {1,2,4,8}", pl.k);
   if (pl.warps < 1 || pl.warps > 8) return fail(c, WF_EINVAL, "warps=%d out of range 1..8", pl.warps);
   if (pl.skew < 1 || pl.skew > 4) return fail(c, WF_EINVAL, "skew=%d out of range 1..4", pl.skew);
